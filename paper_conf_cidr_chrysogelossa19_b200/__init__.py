@@ -1,0 +1,176 @@
+"""HAPE radix hash equi-join, B200-native (sm_100a) -- thin Python front end.
+
+The product is libhape.so (csrc/, C ABI in include/hape.h).  This module only
+marshals torch tensors into the ABI structs: it never computes any part of the
+join and has no fallback path.
+
+    from paper_conf_cidr_chrysogelossa19_b200 import RadixJoin
+    j = RadixJoin(key_dtype=torch.int32)
+    res = j.join(rk, rp, sk, sp)            # CUDA tensors (or pinned host tensors)
+    res.match_count, res.sum_r_payload, res.sum_s_payload, res.pair_checksum
+"""
+from __future__ import annotations
+
+import ctypes
+import dataclasses
+from typing import Optional
+
+from . import _lib
+from ._lib import (HAPE_INT32, HAPE_INT64, HAPE_MEM_DEVICE, HAPE_MEM_HOST, HAPE_OK,
+                   HAPE_ERR_OUTPUT_CAPACITY, HAPE_PART_HASH, HAPE_PART_IDENTITY, STAGES,
+                   hape_join_config, hape_join_create, hape_join_destroy, hape_join_plan,
+                   hape_join_result, hape_last_error, hape_output, hape_radix_join,
+                   hape_relation, hape_status_string, hape_debug_partition, hape_version)
+
+__all__ = ["RadixJoin", "JoinResult", "HapeError", "hape_version", "hape_join_create",
+           "hape_radix_join", "hape_join_destroy", "STAGES"]
+
+
+class HapeError(RuntimeError):
+    def __init__(self, status: int, detail: str):
+        super().__init__(f"{hape_status_string(status)}: {detail}")
+        self.status = status
+
+
+@dataclasses.dataclass
+class JoinResult:
+    status: int
+    match_count: int
+    sum_r_payload: int
+    sum_s_payload: int
+    pair_checksum: int
+    local_match_count: int
+    local_sum_r: int
+    local_sum_s: int
+    local_pair_checksum: int
+    n_written: int
+    n_required: int
+    r_local: int
+    s_local: int
+    passes: int
+    bits: tuple
+    n_partitions: int
+    n_items: int
+    kernel_launches: int
+    stage_ms: dict
+
+    def as_tuple(self):
+        return (self.match_count, self.sum_r_payload, self.sum_s_payload, self.pair_checksum)
+
+
+def _dt(torch_dtype) -> int:
+    import torch
+    if torch_dtype == torch.int32:
+        return HAPE_INT32
+    if torch_dtype == torch.int64:
+        return HAPE_INT64
+    raise TypeError(f"unsupported dtype {torch_dtype} (int32 / int64 only)")
+
+
+def _rel(key, pay) -> hape_relation:
+    if key.dim() != 1 or pay.dim() != 1 or key.shape[0] != pay.shape[0]:
+        raise ValueError("key/payload must be 1-D columns of equal length")
+    if not key.is_contiguous() or not pay.is_contiguous():
+        raise ValueError("columns must be contiguous")
+    if key.device.type != pay.device.type:
+        raise ValueError("key and payload must live on the same device type")
+    mem = HAPE_MEM_DEVICE if key.is_cuda else HAPE_MEM_HOST
+    return hape_relation(key.data_ptr() if key.numel() else None,
+                         pay.data_ptr() if pay.numel() else None, key.shape[0], mem)
+
+
+class RadixJoin:
+    """Owns one hape_join handle (one per process and device)."""
+
+    def __init__(self, key_dtype=None, r_payload_dtype=None, s_payload_dtype=None, device: int = 0,
+                 radix_passes: int = 0, radix_bits=(0, 0), identity: bool = False,
+                 max_r: int = 0, max_s: int = 0, world_size: int = 1, rank: int = 0,
+                 nccl_comm=None, stream=None):
+        import torch
+        key_dtype = key_dtype or torch.int32
+        cfg = hape_join_config()
+        cfg.device = device
+        cfg.key_type = _dt(key_dtype)
+        cfg.r_payload_type = _dt(r_payload_dtype or key_dtype)
+        cfg.s_payload_type = _dt(s_payload_dtype or key_dtype)
+        cfg.radix_passes = radix_passes
+        cfg.radix_bits[0], cfg.radix_bits[1] = radix_bits
+        cfg.part_fn = HAPE_PART_IDENTITY if identity else HAPE_PART_HASH
+        cfg.max_r, cfg.max_s = max_r, max_s
+        cfg.world_size, cfg.rank = world_size, rank
+        cfg.nccl_comm = nccl_comm.value if isinstance(nccl_comm, ctypes.c_void_p) else nccl_comm
+        if stream is not None:
+            cfg.stream = stream.cuda_stream if hasattr(stream, "cuda_stream") else int(stream)
+        self.cfg = cfg
+        st, h = hape_join_create(cfg)
+        if st != HAPE_OK:
+            raise HapeError(st, "hape_join_create failed")
+        self._h = h
+
+    def close(self):
+        if getattr(self, "_h", None) is not None and self._h.value:
+            hape_join_destroy(self._h)
+            self._h = None
+
+    def __del__(self):
+        try:
+            self.close()
+        except Exception:
+            pass
+
+    def __enter__(self):
+        return self
+
+    def __exit__(self, *a):
+        self.close()
+
+    @property
+    def handle(self):
+        return self._h
+
+    def plan(self, n_r: int, n_s: int):
+        st, p = hape_join_plan(self._h, n_r, n_s)
+        if st != HAPE_OK:
+            raise HapeError(st, hape_last_error(self._h))
+        return p
+
+    def join(self, rk, rp, sk, sp, out_r=None, out_s=None, raise_on_capacity: bool = True) -> JoinResult:
+        R = _rel(rk, rp)
+        S = _rel(sk, sp)
+        out = None
+        if out_r is not None:
+            if out_s is None or out_r.shape[0] != out_s.shape[0]:
+                raise ValueError("out_r / out_s must be given together with equal length")
+            out = hape_output(out_r.data_ptr(), out_s.data_ptr(), out_r.shape[0],
+                              HAPE_MEM_DEVICE if out_r.is_cuda else HAPE_MEM_HOST)
+        res = hape_join_result()
+        st = hape_radix_join(self._h, R, S, out, res)
+        if st != HAPE_OK and not (st == HAPE_ERR_OUTPUT_CAPACITY and not raise_on_capacity):
+            raise HapeError(st, hape_last_error(self._h))
+        return JoinResult(
+            status=st, match_count=res.match_count, sum_r_payload=res.sum_r_payload,
+            sum_s_payload=res.sum_s_payload, pair_checksum=res.pair_checksum,
+            local_match_count=res.local_match_count, local_sum_r=res.local_sum_r,
+            local_sum_s=res.local_sum_s, local_pair_checksum=res.local_pair_checksum,
+            n_written=res.n_written, n_required=res.n_required, r_local=res.r_local,
+            s_local=res.s_local, passes=res.passes, bits=(res.bits[0], res.bits[1]),
+            n_partitions=res.n_partitions, n_items=res.n_items,
+            kernel_launches=res.kernel_launches,
+            stage_ms={name: float(res.stage_ms[i]) for i, name in enumerate(STAGES)})
+
+    def debug_partition(self, key, pay, is_s: bool = False, plan=None):
+        """Run the planned radix passes on one relation; returns
+        (partitioned keys, partitioned payloads, bounds[int64], plan)."""
+        import torch
+        rel = _rel(key, pay)
+        dev = torch.device("cuda", self.cfg.device)
+        ok = torch.empty_like(key, device=dev)
+        op = torch.empty_like(pay, device=dev)
+        p = plan or self.plan(key.shape[0], key.shape[0])
+        Q = 1 << (p.bits[0] + (p.bits[1] if p.passes == 2 else 0))
+        ob = torch.empty(Q + 1, dtype=torch.int32, device=dev)
+        st, pout = hape_debug_partition(self._h, rel, int(is_s), p, ok.data_ptr(), op.data_ptr(),
+                                        ob.data_ptr())
+        if st != HAPE_OK:
+            raise HapeError(st, hape_last_error(self._h))
+        return ok, op, ob.to(torch.int64) & 0xFFFFFFFF, pout

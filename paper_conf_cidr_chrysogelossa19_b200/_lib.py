@@ -1,0 +1,189 @@
+"""ctypes binding of include/hape.h -- argument marshalling only.
+
+Function names are the C names.  Every step of the join runs in libhape.so's
+sm_100a kernels; there is no Python or CPU fallback: if the library cannot be
+loaded, importing the binding raises.
+"""
+from __future__ import annotations
+
+import ctypes
+import os
+
+_PKG = os.path.dirname(os.path.abspath(__file__))
+LIB_PATH = os.path.join(_PKG, "libhape.so")
+
+HAPE_OK = 0
+HAPE_ERR_INVALID_ARG = 1
+HAPE_ERR_CUDA = 2
+HAPE_ERR_OOM = 3
+HAPE_ERR_OUTPUT_CAPACITY = 4
+HAPE_ERR_NCCL = 5
+HAPE_ERR_UNSUPPORTED = 6
+
+HAPE_INT32 = 0
+HAPE_INT64 = 1
+HAPE_PART_HASH = 0
+HAPE_PART_IDENTITY = 1
+HAPE_MEM_DEVICE = 0
+HAPE_MEM_HOST = 1
+
+STAGES = ["h2d", "devpart", "exchange", "hist1", "scan1", "scatter1", "hist2", "scan2",
+          "scatter2", "worklist", "build_probe", "finalize", "total"]
+HAPE_NSTAGES = len(STAGES)
+
+EXPORTED = ["hape_version", "hape_status_string", "hape_join_create", "hape_radix_join",
+            "hape_join_destroy", "hape_last_error", "hape_join_plan", "hape_debug_partition",
+            "hape_nccl_unique_id", "hape_nccl_comm_init", "hape_nccl_comm_destroy",
+            "hape_exchange_plan"]
+
+
+class hape_join_config(ctypes.Structure):
+    _fields_ = [("device", ctypes.c_int), ("key_type", ctypes.c_int),
+                ("r_payload_type", ctypes.c_int), ("s_payload_type", ctypes.c_int),
+                ("radix_passes", ctypes.c_int), ("radix_bits", ctypes.c_int * 2),
+                ("part_fn", ctypes.c_int), ("max_r", ctypes.c_uint64), ("max_s", ctypes.c_uint64),
+                ("world_size", ctypes.c_int), ("rank", ctypes.c_int),
+                ("nccl_comm", ctypes.c_void_p), ("stream", ctypes.c_void_p), ("flags", ctypes.c_int)]
+
+
+class hape_relation(ctypes.Structure):
+    _fields_ = [("key", ctypes.c_void_p), ("payload", ctypes.c_void_p), ("n", ctypes.c_uint64),
+                ("mem", ctypes.c_int)]
+
+
+class hape_output(ctypes.Structure):
+    _fields_ = [("r_payload", ctypes.c_void_p), ("s_payload", ctypes.c_void_p),
+                ("capacity", ctypes.c_uint64), ("mem", ctypes.c_int)]
+
+
+class hape_join_result(ctypes.Structure):
+    _fields_ = [("match_count", ctypes.c_uint64), ("sum_r_payload", ctypes.c_uint64),
+                ("sum_s_payload", ctypes.c_uint64), ("pair_checksum", ctypes.c_uint64),
+                ("local_match_count", ctypes.c_uint64), ("local_sum_r", ctypes.c_uint64),
+                ("local_sum_s", ctypes.c_uint64), ("local_pair_checksum", ctypes.c_uint64),
+                ("n_written", ctypes.c_uint64), ("n_required", ctypes.c_uint64),
+                ("r_local", ctypes.c_uint64), ("s_local", ctypes.c_uint64),
+                ("passes", ctypes.c_uint32), ("bits", ctypes.c_uint32 * 2),
+                ("n_partitions", ctypes.c_uint32), ("n_items", ctypes.c_uint32),
+                ("kernel_launches", ctypes.c_uint32), ("stage_ms", ctypes.c_float * HAPE_NSTAGES)]
+
+
+class hape_plan(ctypes.Structure):
+    _fields_ = [("passes", ctypes.c_uint32), ("bits", ctypes.c_uint32 * 2),
+                ("slot_bits", ctypes.c_uint32), ("slot_shift", ctypes.c_uint32),
+                ("dest_bits", ctypes.c_uint32), ("ctas_per_seg", ctypes.c_uint32 * 2),
+                ("build_cap", ctypes.c_uint32), ("probe_slice", ctypes.c_uint32),
+                ("join_ctas", ctypes.c_uint32)]
+
+
+def _load() -> ctypes.CDLL:
+    if not os.path.exists(LIB_PATH):
+        raise ImportError(f"{LIB_PATH} is missing: run __graft_entry__.build() "
+                          "(python -m paper_conf_cidr_chrysogelossa19_b200.build); there is no fallback")
+    lib = ctypes.CDLL(LIB_PATH)
+    P = ctypes.POINTER
+    vp = ctypes.c_void_p
+    lib.hape_version.restype = ctypes.c_char_p
+    lib.hape_version.argtypes = []
+    lib.hape_status_string.restype = ctypes.c_char_p
+    lib.hape_status_string.argtypes = [ctypes.c_int]
+    lib.hape_join_create.restype = ctypes.c_int
+    lib.hape_join_create.argtypes = [P(hape_join_config), P(vp)]
+    lib.hape_radix_join.restype = ctypes.c_int
+    lib.hape_radix_join.argtypes = [vp, P(hape_relation), P(hape_relation), P(hape_output),
+                                    P(hape_join_result)]
+    lib.hape_join_destroy.restype = ctypes.c_int
+    lib.hape_join_destroy.argtypes = [vp]
+    lib.hape_last_error.restype = ctypes.c_char_p
+    lib.hape_last_error.argtypes = [vp]
+    lib.hape_join_plan.restype = ctypes.c_int
+    lib.hape_join_plan.argtypes = [vp, ctypes.c_uint64, ctypes.c_uint64, P(hape_plan)]
+    lib.hape_debug_partition.restype = ctypes.c_int
+    lib.hape_debug_partition.argtypes = [vp, P(hape_relation), ctypes.c_int, P(hape_plan), vp, vp,
+                                         vp, P(hape_plan)]
+    lib.hape_nccl_unique_id.restype = ctypes.c_int
+    lib.hape_nccl_unique_id.argtypes = [vp]
+    lib.hape_nccl_comm_init.restype = ctypes.c_int
+    lib.hape_nccl_comm_init.argtypes = [vp, ctypes.c_int, ctypes.c_int, ctypes.c_int, P(vp)]
+    lib.hape_nccl_comm_destroy.restype = ctypes.c_int
+    lib.hape_nccl_comm_destroy.argtypes = [vp]
+    lib.hape_exchange_plan.restype = ctypes.c_int
+    lib.hape_exchange_plan.argtypes = [ctypes.c_int, ctypes.c_int, P(ctypes.c_uint64),
+                                       P(ctypes.c_uint64), P(ctypes.c_uint64), P(ctypes.c_uint64)]
+    return lib
+
+
+lib = _load()
+
+
+# -- same names as the C ABI ------------------------------------------------
+def hape_version() -> str:
+    return lib.hape_version().decode()
+
+
+def hape_status_string(s: int) -> str:
+    return lib.hape_status_string(s).decode()
+
+
+def hape_join_create(cfg: hape_join_config):
+    h = ctypes.c_void_p()
+    st = lib.hape_join_create(ctypes.byref(cfg), ctypes.byref(h))
+    return st, h
+
+
+def hape_radix_join(h, R: hape_relation, S: hape_relation, out, res: hape_join_result) -> int:
+    return lib.hape_radix_join(h, ctypes.byref(R), ctypes.byref(S),
+                               ctypes.byref(out) if out is not None else None, ctypes.byref(res))
+
+
+def hape_join_destroy(h) -> int:
+    return lib.hape_join_destroy(h)
+
+
+def hape_last_error(h) -> str:
+    r = lib.hape_last_error(h)
+    return r.decode() if r else ""
+
+
+def hape_join_plan(h, n_r: int, n_s: int):
+    p = hape_plan()
+    st = lib.hape_join_plan(h, n_r, n_s, ctypes.byref(p))
+    return st, p
+
+
+def hape_debug_partition(h, rel: hape_relation, is_s: int, plan_in, out_keys: int,
+                         out_payloads: int, out_bounds: int):
+    p = hape_plan()
+    st = lib.hape_debug_partition(h, ctypes.byref(rel), is_s,
+                                  ctypes.byref(plan_in) if plan_in is not None else None,
+                                  out_keys, out_payloads, out_bounds, ctypes.byref(p))
+    return st, p
+
+
+def hape_nccl_unique_id() -> bytes:
+    buf = ctypes.create_string_buffer(128)
+    st = lib.hape_nccl_unique_id(buf)
+    if st != HAPE_OK:
+        raise RuntimeError(hape_status_string(st))
+    return buf.raw
+
+
+def hape_nccl_comm_init(uid: bytes, world: int, rank: int, device: int):
+    comm = ctypes.c_void_p()
+    buf = ctypes.create_string_buffer(uid, 128)
+    st = lib.hape_nccl_comm_init(buf, world, rank, device, ctypes.byref(comm))
+    return st, comm
+
+
+def hape_nccl_comm_destroy(comm) -> int:
+    return lib.hape_nccl_comm_destroy(comm)
+
+
+def hape_exchange_plan(world: int, rank: int, counts):
+    G = world
+    c = (ctypes.c_uint64 * (G * G))(*[int(x) for x in counts])
+    so = (ctypes.c_uint64 * G)()
+    ro = (ctypes.c_uint64 * G)()
+    rt = ctypes.c_uint64()
+    st = lib.hape_exchange_plan(G, rank, c, so, ro, ctypes.byref(rt))
+    return st, list(so), list(ro), int(rt.value)

@@ -1,0 +1,862 @@
+// hape.cu -- C ABI (include/hape.h) and host orchestration of the radix join.
+//
+// Stage sequence of one hape_radix_join call (e):
+//   [H2D staging]                         host-resident inputs only
+//   [device partition + exchange]         G>1: route by top log2(G) bits of h
+//                                         (HetExchange hash router + mem-move,
+//                                         PAPER.md P643-656, P717-737)
+//   pass 1: hist -> scan -> scatter       (a6-a8; P572-598, Fig. 4)
+//   pass 2: the same inside each pass-1 partition  (a9; P140-145, P589-593)
+//   work list -> build+probe+aggregate    (a10-a12; P535-541, Fig. 3, P789-793)
+//   result D2H (+ NCCL allreduce)         (a13)
+// Every stage is one or two kernel launches on the handle's stream; the only
+// host synchronisation points are the count exchange (G>1) and the result.
+#include <cuda_runtime.h>
+#include <nccl.h>
+
+#include <algorithm>
+#include <cstdarg>
+#include <cstdio>
+#include <cstring>
+#include <string>
+#include <vector>
+
+#include "hape.h"
+#include "kernels.cuh"
+
+using namespace hape;
+
+namespace {
+
+struct DevBuf {
+  void* p = nullptr;
+  size_t bytes = 0;
+};
+
+constexpr uint32_t kTargetPerPartition = 2048;  // R tuples per co-partition (Fig. 5 range, P753-858)
+constexpr uint32_t kMaxBitsPerPass = 12;
+constexpr uint32_t kMaxSinglePassBits = 10;
+constexpr uint32_t kChunk = 32768;              // tuples per partitioning CTA (upper bound)
+constexpr uint32_t kMinChunk = 1024;
+
+inline uint32_t ceil_log2_u64(uint64_t x) {
+  uint32_t b = 0;
+  while ((1ull << b) < x) b++;
+  return b;
+}
+
+}  // namespace
+
+struct hape_join {
+  hape_join_config cfg{};
+  int dev = 0;
+  int num_sms = 148;
+  cudaStream_t stream = nullptr;
+  bool own_stream = false;
+  ncclComm_t comm = nullptr;
+  std::string err;
+  cudaEvent_t ev[HAPE_NSTAGES + 1] = {};
+  bool ev_used[HAPE_NSTAGES] = {};
+  uint32_t launches = 0;
+  // workspace
+  DevBuf stage[4];        // host-input staging: R key, R pay, S key, S pay
+  DevBuf ping[4];         // pass-1 output
+  DevBuf pong[4];         // pass-2 output
+  DevBuf send[4];         // G>1 device-partition output
+  DevBuf recv[4];         // G>1 exchange receive buffers
+  DevBuf outst[2];        // host-output staging
+  DevBuf small;           // histograms, bounds, work list, counters
+  unsigned long long* h_res = nullptr;  // pinned: acc[4], out_ctr, (n_items | item_ctr)
+  uint32_t* h_bounds = nullptr;         // pinned: gathered device-partition bounds
+  size_t h_bounds_cap = 0;
+};
+
+// ---------------------------------------------------------------------------
+// error plumbing
+// ---------------------------------------------------------------------------
+static hape_status fail(hape_join* h, hape_status s, const char* fmt, ...) {
+  if (h) {
+    char buf[512];
+    va_list ap;
+    va_start(ap, fmt);
+    vsnprintf(buf, sizeof buf, fmt, ap);
+    va_end(ap);
+    h->err = buf;
+  }
+  return s;
+}
+
+#define CK(h, call)                                                                      \
+  do {                                                                                   \
+    cudaError_t e_ = (call);                                                             \
+    if (e_ != cudaSuccess) {                                                             \
+      (void)cudaGetLastError();                                                          \
+      return fail((h), e_ == cudaErrorMemoryAllocation ? HAPE_ERR_OOM : HAPE_ERR_CUDA,   \
+                  "%s:%d %s: %s", __FILE__, __LINE__, #call, cudaGetErrorString(e_));    \
+    }                                                                                    \
+  } while (0)
+
+#define CKN(h, call)                                                                     \
+  do {                                                                                   \
+    ncclResult_t r_ = (call);                                                            \
+    if (r_ != ncclSuccess)                                                               \
+      return fail((h), HAPE_ERR_NCCL, "%s:%d %s: %s", __FILE__, __LINE__, #call,         \
+                  ncclGetErrorString(r_));                                               \
+  } while (0)
+
+#define CKS(call)                         \
+  do {                                    \
+    hape_status s_ = (call);              \
+    if (s_ != HAPE_OK) return s_;         \
+  } while (0)
+
+#define CK_LAUNCH(h)                                                                     \
+  do {                                                                                   \
+    (h)->launches++;                                                                     \
+    CK(h, cudaGetLastError());                                                           \
+  } while (0)
+
+static hape_status ensure(hape_join* h, DevBuf& b, size_t bytes) {
+  if (bytes <= b.bytes) return HAPE_OK;
+  if (b.p) {
+    CK(h, cudaStreamSynchronize(h->stream));
+    CK(h, cudaFree(b.p));
+    b.p = nullptr;
+    b.bytes = 0;
+  }
+  size_t want = (bytes + 4095) & ~(size_t)4095;
+  cudaError_t e = cudaMalloc(&b.p, want);
+  if (e != cudaSuccess) {
+    (void)cudaGetLastError();
+    b.p = nullptr;
+    return fail(h, HAPE_ERR_OOM, "cudaMalloc(%zu) failed: %s", want, cudaGetErrorString(e));
+  }
+  b.bytes = want;
+  return HAPE_OK;
+}
+
+static void mark(hape_join* h, int stage) {
+  cudaEventRecord(h->ev[stage], h->stream);
+  h->ev_used[stage] = true;
+}
+
+// ---------------------------------------------------------------------------
+// plan (a1): bits per pass, co-partition capacity, CTA shapes
+// ---------------------------------------------------------------------------
+static int key_width(const hape_join_config& c) { return c.key_type == HAPE_INT64 ? 8 : 4; }
+static int pay_width(hape_dtype t) { return t == HAPE_INT64 ? 8 : 4; }
+
+static uint32_t cps_for(const hape_join* h, uint64_t total, uint32_t nseg) {
+  const uint64_t avg = nseg ? (total + nseg - 1) / nseg : total;
+  uint64_t c = (avg + kChunk - 1) / kChunk;
+  const uint64_t want_ctas = (uint64_t)h->num_sms * 8;
+  if (c * nseg < want_ctas) {
+    uint64_t c2 = (want_ctas + nseg - 1) / nseg;
+    uint64_t cmax = std::max<uint64_t>(1, (avg + kMinChunk - 1) / kMinChunk);
+    c = std::max<uint64_t>(c, std::min(c2, cmax));
+  }
+  return (uint32_t)std::max<uint64_t>(1, std::min<uint64_t>(c, 1u << 20));
+}
+
+static hape_status make_plan(const hape_join* h, uint64_t n_r, uint64_t n_s, hape_plan* p) {
+  const hape_join_config& c = h->cfg;
+  memset(p, 0, sizeof *p);
+  const uint32_t HW = key_width(c) * 8;
+  const int world = c.world_size > 1 ? c.world_size : 1;
+  p->dest_bits = ceil_log2_u64((uint64_t)world);
+  uint32_t need = 0;
+  while ((n_r >> need) > kTargetPerPartition) need++;
+  uint32_t passes = c.radix_passes ? (uint32_t)c.radix_passes : (need <= kMaxSinglePassBits ? 1u : 2u);
+  uint32_t b1, b2;
+  if (c.radix_bits[0] > 0) {
+    b1 = (uint32_t)c.radix_bits[0];
+    b2 = passes == 2 ? (uint32_t)std::max(0, c.radix_bits[1]) : 0u;
+  } else if (passes == 1) {
+    b1 = std::min(need, kMaxBitsPerPass);
+    b2 = 0;
+  } else {
+    b1 = std::min((need + 1) / 2, kMaxBitsPerPass);
+    b2 = std::min(need - std::min(need, b1), kMaxBitsPerPass);
+  }
+  if (b1 > kMaxBitsPerPass || b2 > kMaxBitsPerPass) return HAPE_ERR_INVALID_ARG;
+  if (b1 + b2 + p->dest_bits > HW) return HAPE_ERR_INVALID_ARG;
+  p->passes = passes;
+  p->bits[0] = b1;
+  p->bits[1] = b2;
+  const uint64_t Q = 1ull << (b1 + b2);
+  const uint64_t expected = (n_r + Q - 1) / Q;
+  uint64_t cap = expected + expected / 4 + 128;
+  cap = std::max<uint64_t>(512, std::min<uint64_t>(cap, 8192));
+  cap = (cap + 255) & ~255ull;
+  p->build_cap = (uint32_t)cap;
+  uint32_t sb = ceil_log2_u64(cap);
+  sb = std::max(6u, std::min(sb, 14u));
+  p->slot_shift = b1 + b2;
+  const int avail = (int)HW - (int)p->dest_bits - (int)p->slot_shift;
+  if ((int)sb > avail) sb = (uint32_t)std::max(0, avail);
+  p->slot_bits = sb;
+  p->probe_slice = 16384;
+  p->ctas_per_seg[0] = cps_for(h, n_r, 1);
+  p->ctas_per_seg[1] = passes == 2 ? cps_for(h, n_r, 1u << b1) : 0;
+  p->join_ctas = 0;  // filled at launch (occupancy)
+  return HAPE_OK;
+}
+
+// ---------------------------------------------------------------------------
+// kernel launchers (dtype dispatch)
+// ---------------------------------------------------------------------------
+struct Col {
+  const void* k;
+  const void* p;
+  uint32_t n;
+  int pw;
+};
+
+static hape_status launch_hist(hape_join* h, int kw, const void* key, SegMap m, BitField bf, uint32_t P,
+                               uint32_t* hist, uint32_t* rowsum) {
+  const unsigned grid = m.nseg * m.cps;
+  const size_t smem = (size_t)P * 4;
+  const int ident = h->cfg.part_fn == HAPE_PART_IDENTITY;
+  if (grid == 0) return HAPE_OK;
+  if (kw == 4)
+    k_hist<4><<<grid, HIST_THREADS, smem, h->stream>>>((const uint32_t*)key, m, bf, ident, P, hist, rowsum);
+  else
+    k_hist<8><<<grid, HIST_THREADS, smem, h->stream>>>((const uint64_t*)key, m, bf, ident, P, hist, rowsum);
+  CK_LAUNCH(h);
+  return HAPE_OK;
+}
+
+static hape_status launch_scan(hape_join* h, SegMap m, uint32_t P, uint32_t* hist, const uint32_t* rowsum,
+                               uint32_t* bounds_out) {
+  uint32_t rpc = std::max<uint32_t>(1, SCAN_TILE / m.cps);
+  rpc = std::min(rpc, P);
+  const uint32_t groups = (P + rpc - 1) / rpc;
+  k_scan<<<m.nseg * groups, SCAN_THREADS, 0, h->stream>>>(hist, rowsum, m, P, rpc, bounds_out);
+  CK_LAUNCH(h);
+  return HAPE_OK;
+}
+
+template <int KW, int PW>
+static hape_status launch_scatter_t(hape_join* h, const Col& in, SegMap m, BitField bf, uint32_t P,
+                                    const uint32_t* offs, void* ok, void* op) {
+  const size_t smem = scatter_smem_bytes<KW, PW>(P);
+  static bool attr_set = false;
+  if (!attr_set) {
+    CK(h, cudaFuncSetAttribute(k_scatter<KW, PW>, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024));
+    attr_set = true;
+  }
+  const unsigned grid = m.nseg * m.cps;
+  if (grid == 0) return HAPE_OK;
+  k_scatter<KW, PW><<<grid, SC_THREADS, smem, h->stream>>>(
+      (const typename UW<KW>::T*)in.k, (const typename UW<PW>::T*)in.p, m, bf,
+      h->cfg.part_fn == HAPE_PART_IDENTITY, P, offs, (typename UW<KW>::T*)ok, (typename UW<PW>::T*)op);
+  CK_LAUNCH(h);
+  return HAPE_OK;
+}
+
+static hape_status launch_scatter(hape_join* h, int kw, const Col& in, SegMap m, BitField bf, uint32_t P,
+                                  const uint32_t* offs, void* ok, void* op) {
+  if (kw == 4 && in.pw == 4) return launch_scatter_t<4, 4>(h, in, m, bf, P, offs, ok, op);
+  if (kw == 4 && in.pw == 8) return launch_scatter_t<4, 8>(h, in, m, bf, P, offs, ok, op);
+  if (kw == 8 && in.pw == 4) return launch_scatter_t<8, 4>(h, in, m, bf, P, offs, ok, op);
+  return launch_scatter_t<8, 8>(h, in, m, bf, P, offs, ok, op);
+}
+
+template <int KW, int PRW, int PSW, bool MAT>
+static hape_status launch_join_t(hape_join* h, const JoinArgs& a, uint32_t* ctas_out) {
+  auto kern = k_build_probe<KW, PRW, PSW, MAT>;
+  const size_t smem = join_smem_bytes<KW, PRW, PSW>(a.cap, a.slot_bits);
+  static bool attr_set = false;
+  if (!attr_set) {
+    CK(h, cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024));
+    attr_set = true;
+  }
+  int per_sm = 0;
+  CK(h, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, JN_THREADS, smem));
+  if (per_sm < 1) return fail(h, HAPE_ERR_UNSUPPORTED, "build+probe does not fit: smem %zu", smem);
+  const unsigned grid = (unsigned)(per_sm * h->num_sms);
+  *ctas_out = grid;
+  kern<<<grid, JN_THREADS, smem, h->stream>>>(a);
+  CK_LAUNCH(h);
+  return HAPE_OK;
+}
+
+template <int KW, int PRW, int PSW>
+static hape_status launch_join_m(hape_join* h, const JoinArgs& a, bool mat, uint32_t* ctas) {
+  return mat ? launch_join_t<KW, PRW, PSW, true>(h, a, ctas) : launch_join_t<KW, PRW, PSW, false>(h, a, ctas);
+}
+
+static hape_status launch_join(hape_join* h, int kw, int prw, int psw, const JoinArgs& a, bool mat,
+                               uint32_t* ctas) {
+  if (kw == 4) {
+    if (prw == 4) return psw == 4 ? launch_join_m<4, 4, 4>(h, a, mat, ctas) : launch_join_m<4, 4, 8>(h, a, mat, ctas);
+    return psw == 4 ? launch_join_m<4, 8, 4>(h, a, mat, ctas) : launch_join_m<4, 8, 8>(h, a, mat, ctas);
+  }
+  if (prw == 4) return psw == 4 ? launch_join_m<8, 4, 4>(h, a, mat, ctas) : launch_join_m<8, 4, 8>(h, a, mat, ctas);
+  return psw == 4 ? launch_join_m<8, 8, 4>(h, a, mat, ctas) : launch_join_m<8, 8, 8>(h, a, mat, ctas);
+}
+
+// ---------------------------------------------------------------------------
+// small-buffer carve-up for one call
+// ---------------------------------------------------------------------------
+struct Carve {
+  size_t off = 0;
+  size_t take(size_t bytes) {
+    size_t o = (off + 255) & ~(size_t)255;
+    off = o + bytes;
+    return o;
+  }
+};
+
+struct SideLayout {            // per relation
+  uint32_t cps1 = 0, cps2 = 0;
+  size_t hist1 = 0, rowsum1 = 0, bounds1 = 0, hist2 = 0, rowsum2 = 0, bounds2 = 0;
+};
+
+struct CallLayout {
+  size_t zero_lo = 0, zero_hi = 0;
+  size_t acc = 0, out_ctr = 0, ctrs = 0, items = 0;
+  SideLayout side[2];
+  size_t total = 0;
+  uint32_t n_items_cap = 0;
+};
+
+static CallLayout layout_for(const hape_join* h, const hape_plan& pl, uint64_t n_r, uint64_t n_s) {
+  CallLayout L;
+  Carve cv;
+  const uint64_t P1 = 1ull << pl.bits[0], P2 = pl.passes == 2 ? (1ull << pl.bits[1]) : 1ull;
+  const uint64_t Q = P1 * P2;
+  // zeroed region first: acc[4] u64, out_ctr u64, ctrs (n_items, item_ctr), rowsums
+  L.acc = cv.take(4 * 8);
+  L.zero_lo = L.acc;
+  L.out_ctr = cv.take(8);
+  L.ctrs = cv.take(8);
+  const uint64_t ns[2] = {n_r, n_s};
+  for (int s = 0; s < 2; s++) {
+    L.side[s].rowsum1 = cv.take(P1 * 4);
+    if (pl.passes == 2) L.side[s].rowsum2 = cv.take(Q * 4);
+  }
+  L.zero_hi = cv.off;
+  for (int s = 0; s < 2; s++) {
+    SideLayout& S = L.side[s];
+    S.cps1 = cps_for(h, ns[s], 1);
+    S.hist1 = cv.take(P1 * S.cps1 * 4);
+    S.bounds1 = cv.take((P1 + 1) * 4);
+    if (pl.passes == 2) {
+      S.cps2 = cps_for(h, ns[s], (uint32_t)P1);
+      S.hist2 = cv.take(Q * S.cps2 * 4);
+      S.bounds2 = cv.take((Q + 1) * 4);
+    }
+  }
+  L.n_items_cap = (uint32_t)std::min<uint64_t>(Q + (n_s + pl.probe_slice - 1) / pl.probe_slice + 1, 0xFFFFFFFFu);
+  L.items = cv.take((size_t)L.n_items_cap * 8);
+  L.total = cv.off;
+  return L;
+}
+
+template <class T>
+static T* at(hape_join* h, size_t off) {
+  return reinterpret_cast<T*>(static_cast<char*>(h->small.p) + off);
+}
+
+// Radix passes over one relation: in -> (ping, pong) -> final columns + bounds.
+// Launches are grouped by stage across both relations by the caller.
+struct PassIO {
+  Col in;                      // pass-1 input
+  void* p1k; void* p1p;        // pass-1 output
+  void* p2k; void* p2p;        // pass-2 output
+};
+
+static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const CallLayout& L, PassIO io[2],
+                                        int nside, const void** fin_k, const void** fin_p,
+                                        const uint32_t** fin_bounds) {
+  const int kw = key_width(h->cfg);
+  const uint32_t P1 = 1u << pl.bits[0], P2 = 1u << pl.bits[1];
+  const BitField bf1{0u, P1 - 1}, bf2{pl.bits[0], P2 - 1};
+  SegMap m1[2], m2[2];
+  for (int s = 0; s < nside; s++) {
+    m1[s] = SegMap{nullptr, 1u, L.side[s].cps1, io[s].in.n};
+    if (pl.passes == 2) m2[s] = SegMap{at<uint32_t>(h, L.side[s].bounds1), P1, L.side[s].cps2, io[s].in.n};
+  }
+  mark(h, HAPE_STAGE_HIST1);
+  for (int s = 0; s < nside; s++)
+    CKS(launch_hist(h, kw, io[s].in.k, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1),
+                    at<uint32_t>(h, L.side[s].rowsum1)));
+  mark(h, HAPE_STAGE_SCAN1);
+  for (int s = 0; s < nside; s++)
+    CKS(launch_scan(h, m1[s], P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1),
+                    at<uint32_t>(h, L.side[s].bounds1)));
+  mark(h, HAPE_STAGE_SCATTER1);
+  for (int s = 0; s < nside; s++)
+    CKS(launch_scatter(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), io[s].p1k, io[s].p1p));
+  for (int s = 0; s < nside; s++) {
+    fin_k[s] = io[s].p1k;
+    fin_p[s] = io[s].p1p;
+    fin_bounds[s] = at<uint32_t>(h, L.side[s].bounds1);
+  }
+  if (pl.passes == 2) {
+    mark(h, HAPE_STAGE_HIST2);
+    for (int s = 0; s < nside; s++)
+      CKS(launch_hist(h, kw, io[s].p1k, m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2),
+                      at<uint32_t>(h, L.side[s].rowsum2)));
+    mark(h, HAPE_STAGE_SCAN2);
+    for (int s = 0; s < nside; s++)
+      CKS(launch_scan(h, m2[s], P2, at<uint32_t>(h, L.side[s].hist2), at<uint32_t>(h, L.side[s].rowsum2),
+                      at<uint32_t>(h, L.side[s].bounds2)));
+    mark(h, HAPE_STAGE_SCATTER2);
+    for (int s = 0; s < nside; s++) {
+      Col c2{io[s].p1k, io[s].p1p, io[s].in.n, io[s].in.pw};
+      CKS(launch_scatter(h, kw, c2, m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), io[s].p2k, io[s].p2p));
+      fin_k[s] = io[s].p2k;
+      fin_p[s] = io[s].p2p;
+      fin_bounds[s] = at<uint32_t>(h, L.side[s].bounds2);
+    }
+  }
+  return HAPE_OK;
+}
+
+// ---------------------------------------------------------------------------
+// argument checks
+// ---------------------------------------------------------------------------
+static hape_status check_rel(hape_join* h, const hape_relation* r, int kw, int pw, const char* name) {
+  if (!r) return fail(h, HAPE_ERR_INVALID_ARG, "%s is NULL", name);
+  if (r->n >= 0xFFFFFFFFull) return fail(h, HAPE_ERR_UNSUPPORTED, "%s.n >= 2^32 per rank", name);
+  if (r->mem != HAPE_MEM_DEVICE && r->mem != HAPE_MEM_HOST)
+    return fail(h, HAPE_ERR_INVALID_ARG, "%s.mem invalid", name);
+  if (r->n && (!r->key || !r->payload)) return fail(h, HAPE_ERR_INVALID_ARG, "%s has NULL column with n>0", name);
+  if (((uintptr_t)r->key % kw) || ((uintptr_t)r->payload % pw))
+    return fail(h, HAPE_ERR_INVALID_ARG, "%s column not element-aligned", name);
+  return HAPE_OK;
+}
+
+static hape_status stage_in(hape_join* h, const hape_relation* r, int kw, int pw, DevBuf& bk, DevBuf& bp,
+                            Col* out) {
+  out->n = (uint32_t)r->n;
+  out->pw = pw;
+  if (r->mem == HAPE_MEM_DEVICE || r->n == 0) {
+    out->k = r->key;
+    out->p = r->payload;
+    return HAPE_OK;
+  }
+  CKS(ensure(h, bk, r->n * kw));
+  CKS(ensure(h, bp, r->n * pw));
+  CK(h, cudaMemcpyAsync(bk.p, r->key, r->n * kw, cudaMemcpyHostToDevice, h->stream));
+  CK(h, cudaMemcpyAsync(bp.p, r->payload, r->n * pw, cudaMemcpyHostToDevice, h->stream));
+  out->k = bk.p;
+  out->p = bp.p;
+  return HAPE_OK;
+}
+
+// ---------------------------------------------------------------------------
+// G>1: device partition by destination + NCCL exchange (a2-a5)
+// ---------------------------------------------------------------------------
+extern "C" hape_status hape_exchange_plan(int world_size, int rank, const uint64_t* counts, uint64_t* send_off,
+                                          uint64_t* recv_off, uint64_t* recv_total) {
+  if (world_size < 1 || rank < 0 || rank >= world_size || !counts || !send_off || !recv_off || !recv_total)
+    return HAPE_ERR_INVALID_ARG;
+  const int G = world_size;
+  uint64_t s = 0;
+  for (int d = 0; d < G; d++) { send_off[d] = s; s += counts[(size_t)rank * G + d]; }
+  uint64_t r = 0;
+  for (int src = 0; src < G; src++) { recv_off[src] = r; r += counts[(size_t)src * G + rank]; }
+  *recv_total = r;
+  return HAPE_OK;
+}
+
+static hape_status exchange(hape_join* h, Col in[2], Col out[2]) {
+  const int G = h->cfg.world_size, me = h->cfg.rank;
+  const int kw = key_width(h->cfg);
+  const uint32_t g = ceil_log2_u64((uint64_t)G);
+  const uint32_t HW = kw * 8;
+  const BitField bf{HW - g, (uint32_t)G - 1};
+  // layout in small: per side hist[G*cps], rowsum[G], and the local bounds block [2][G+1] + gathered [G][2][G+1]
+  Carve cv;
+  uint32_t cps[2];
+  size_t hist_off[2], rs_off[2];
+  for (int s = 0; s < 2; s++) {
+    cps[s] = cps_for(h, in[s].n, 1);
+    hist_off[s] = cv.take((size_t)G * cps[s] * 4);
+    rs_off[s] = cv.take((size_t)G * 4);
+  }
+  const size_t bl_off = cv.take((size_t)2 * (G + 1) * 4);
+  const size_t bg_off = cv.take((size_t)G * 2 * (G + 1) * 4);
+  CKS(ensure(h, h->small, cv.off));
+  CK(h, cudaMemsetAsync(at<char>(h, rs_off[0]), 0, (size_t)G * 4, h->stream));
+  CK(h, cudaMemsetAsync(at<char>(h, rs_off[1]), 0, (size_t)G * 4, h->stream));
+  mark(h, HAPE_STAGE_DEVPART);
+  for (int s = 0; s < 2; s++) {
+    CKS(ensure(h, h->send[2 * s], (size_t)in[s].n * kw + 16));
+    CKS(ensure(h, h->send[2 * s + 1], (size_t)in[s].n * in[s].pw + 16));
+    SegMap m{nullptr, 1u, cps[s], in[s].n};
+    uint32_t* hist = at<uint32_t>(h, hist_off[s]);
+    uint32_t* rs = at<uint32_t>(h, rs_off[s]);
+    uint32_t* bl = at<uint32_t>(h, bl_off) + s * (G + 1);
+    CKS(launch_hist(h, kw, in[s].k, m, bf, (uint32_t)G, hist, rs));
+    CKS(launch_scan(h, m, (uint32_t)G, hist, rs, bl));
+    CKS(launch_scatter(h, kw, in[s], m, bf, (uint32_t)G, hist, h->send[2 * s].p, h->send[2 * s + 1].p));
+  }
+  mark(h, HAPE_STAGE_EXCHANGE);
+  // count exchange: all-gather every rank's destination bounds
+  CKN(h, ncclAllGather(at<uint32_t>(h, bl_off), at<uint32_t>(h, bg_off), (size_t)2 * (G + 1), ncclUint32, h->comm,
+                       h->stream));
+  const size_t nb = (size_t)G * 2 * (G + 1);
+  if (h->h_bounds_cap < nb) {
+    if (h->h_bounds) cudaFreeHost(h->h_bounds);
+    CK(h, cudaMallocHost(&h->h_bounds, nb * 4));
+    h->h_bounds_cap = nb;
+  }
+  CK(h, cudaMemcpyAsync(h->h_bounds, at<uint32_t>(h, bg_off), nb * 4, cudaMemcpyDeviceToHost, h->stream));
+  CK(h, cudaStreamSynchronize(h->stream));
+  for (int s = 0; s < 2; s++) {
+    std::vector<uint64_t> counts((size_t)G * G), soff(G), roff(G);
+    for (int src = 0; src < G; src++) {
+      const uint32_t* b = h->h_bounds + (size_t)src * 2 * (G + 1) + s * (G + 1);
+      for (int d = 0; d < G; d++) counts[(size_t)src * G + d] = b[d + 1] - b[d];
+    }
+    uint64_t rtot = 0;
+    hape_exchange_plan(G, me, counts.data(), soff.data(), roff.data(), &rtot);
+    if (rtot >= 0xFFFFFFFFull) return fail(h, HAPE_ERR_UNSUPPORTED, "received %llu tuples >= 2^32", (unsigned long long)rtot);
+    const size_t w[2] = {(size_t)kw, (size_t)in[s].pw};
+    for (int c = 0; c < 2; c++) CKS(ensure(h, h->recv[2 * s + c], rtot * w[c] + 16));
+    CKN(h, ncclGroupStart());
+    for (int c = 0; c < 2; c++) {
+      const char* sb = static_cast<const char*>(h->send[2 * s + c].p);
+      char* rb = static_cast<char*>(h->recv[2 * s + c].p);
+      for (int p = 0; p < G; p++) {
+        const uint64_t sc = counts[(size_t)me * G + p], rc = counts[(size_t)p * G + me];
+        if (sc) CKN(h, ncclSend(sb + soff[p] * w[c], sc * w[c], ncclUint8, p, h->comm, h->stream));
+        if (rc) CKN(h, ncclRecv(rb + roff[p] * w[c], rc * w[c], ncclUint8, p, h->comm, h->stream));
+      }
+    }
+    CKN(h, ncclGroupEnd());
+    out[s] = Col{h->recv[2 * s].p, h->recv[2 * s + 1].p, (uint32_t)rtot, in[s].pw};
+  }
+  return HAPE_OK;
+}
+
+// ---------------------------------------------------------------------------
+// the join
+// ---------------------------------------------------------------------------
+static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_relation* S, const hape_output* out,
+                             hape_join_result* res) {
+  const hape_join_config& c = h->cfg;
+  const int kw = key_width(c), prw = pay_width(c.r_payload_type), psw = pay_width(c.s_payload_type);
+  CKS(check_rel(h, R, kw, prw, "R"));
+  CKS(check_rel(h, S, kw, psw, "S"));
+  const bool mat = out && out->capacity > 0;
+  if (mat) {
+    if (!out->r_payload || !out->s_payload) return fail(h, HAPE_ERR_INVALID_ARG, "output buffers NULL");
+    if (out->mem != HAPE_MEM_DEVICE && out->mem != HAPE_MEM_HOST) return fail(h, HAPE_ERR_INVALID_ARG, "out.mem");
+  }
+  CK(h, cudaSetDevice(h->dev));
+  memset(res, 0, sizeof *res);
+  for (int i = 0; i < HAPE_NSTAGES; i++) h->ev_used[i] = false;
+  h->launches = 0;
+  const int world = c.world_size > 1 ? c.world_size : 1;
+
+  mark(h, HAPE_STAGE_TOTAL);
+  mark(h, HAPE_STAGE_H2D);
+  Col in[2];
+  CKS(stage_in(h, R, kw, prw, h->stage[0], h->stage[1], &in[0]));
+  CKS(stage_in(h, S, kw, psw, h->stage[2], h->stage[3], &in[1]));
+  Col loc[2] = {in[0], in[1]};
+  if (world > 1) CKS(exchange(h, in, loc));
+
+  hape_plan pl;
+  if (make_plan(h, loc[0].n, loc[1].n, &pl) != HAPE_OK)
+    return fail(h, HAPE_ERR_INVALID_ARG, "invalid radix plan (bits/passes)");
+  const CallLayout L = layout_for(h, pl, loc[0].n, loc[1].n);
+  CKS(ensure(h, h->small, L.total));
+  const uint64_t n_loc[2] = {loc[0].n, loc[1].n};
+  const int pw[2] = {prw, psw};
+  for (int s = 0; s < 2; s++) {
+    CKS(ensure(h, h->ping[2 * s], n_loc[s] * kw + 16));
+    CKS(ensure(h, h->ping[2 * s + 1], n_loc[s] * pw[s] + 16));
+    if (pl.passes == 2) {
+      CKS(ensure(h, h->pong[2 * s], n_loc[s] * kw + 16));
+      CKS(ensure(h, h->pong[2 * s + 1], n_loc[s] * pw[s] + 16));
+    }
+  }
+  void* mat_r = nullptr;
+  void* mat_s = nullptr;
+  if (mat) {
+    mat_r = out->r_payload;
+    mat_s = out->s_payload;
+    if (out->mem == HAPE_MEM_HOST) {
+      CKS(ensure(h, h->outst[0], out->capacity * prw));
+      CKS(ensure(h, h->outst[1], out->capacity * psw));
+      mat_r = h->outst[0].p;
+      mat_s = h->outst[1].p;
+    }
+  }
+  CK(h, cudaMemsetAsync(at<char>(h, L.zero_lo), 0, L.zero_hi - L.zero_lo, h->stream));
+
+  PassIO io[2];
+  for (int s = 0; s < 2; s++)
+    io[s] = PassIO{loc[s], h->ping[2 * s].p, h->ping[2 * s + 1].p, h->pong[2 * s].p, h->pong[2 * s + 1].p};
+  const void* fk[2];
+  const void* fp[2];
+  const uint32_t* fb[2];
+  CKS(run_partition_stages(h, pl, L, io, 2, fk, fp, fb));
+
+  const uint32_t Q = 1u << (pl.bits[0] + (pl.passes == 2 ? pl.bits[1] : 0));
+  uint32_t* ctrs = at<uint32_t>(h, L.ctrs);  // [0] n_items, [1] item_ctr
+  mark(h, HAPE_STAGE_WORKLIST);
+  k_worklist<<<(Q + WL_THREADS - 1) / WL_THREADS, WL_THREADS, 0, h->stream>>>(fb[0], fb[1], Q, pl.probe_slice,
+                                                                              at<uint2>(h, L.items), ctrs);
+  CK_LAUNCH(h);
+
+  mark(h, HAPE_STAGE_BUILD_PROBE);
+  JoinArgs ja{};
+  ja.rk = fk[0]; ja.rp = fp[0]; ja.sk = fk[1]; ja.sp = fp[1];
+  ja.bR = fb[0]; ja.bS = fb[1];
+  ja.items = at<uint2>(h, L.items); ja.n_items = ctrs; ja.item_ctr = ctrs + 1;
+  ja.cap = pl.build_cap; ja.slice = pl.probe_slice; ja.slot_shift = pl.slot_shift; ja.slot_bits = pl.slot_bits;
+  ja.ident = c.part_fn == HAPE_PART_IDENTITY;
+  ja.acc = at<unsigned long long>(h, L.acc);
+  ja.out_r = mat_r; ja.out_s = mat_s; ja.out_cap = mat ? out->capacity : 0;
+  ja.out_ctr = at<unsigned long long>(h, L.out_ctr);
+  CKS(launch_join(h, kw, prw, psw, ja, mat, &pl.join_ctas));
+
+  mark(h, HAPE_STAGE_FINALIZE);
+  // local result: acc[4], out_ctr, ctrs -- contiguous at L.acc (6 x u64)
+  CK(h, cudaMemcpyAsync(h->h_res, at<char>(h, L.acc), 4 * 8, cudaMemcpyDeviceToHost, h->stream));
+  CK(h, cudaMemcpyAsync(h->h_res + 4, at<char>(h, L.out_ctr), 8, cudaMemcpyDeviceToHost, h->stream));
+  CK(h, cudaMemcpyAsync(h->h_res + 5, at<char>(h, L.ctrs), 8, cudaMemcpyDeviceToHost, h->stream));
+  if (world > 1) {
+    // global result: NCCL allreduce (sum, u64, wrapping) of the four fields
+    unsigned long long* acc = at<unsigned long long>(h, L.acc);
+    CKN(h, ncclAllReduce(acc, acc, 4, ncclUint64, ncclSum, h->comm, h->stream));
+    CK(h, cudaMemcpyAsync(h->h_res + 6, acc, 4 * 8, cudaMemcpyDeviceToHost, h->stream));
+  }
+  CK(h, cudaStreamSynchronize(h->stream));
+  const unsigned long long* r = h->h_res;
+  res->local_match_count = r[0];
+  res->local_sum_r = r[1];
+  res->local_sum_s = r[2];
+  res->local_pair_checksum = r[3];
+  const unsigned long long* g = world > 1 ? r + 6 : r;
+  res->match_count = g[0];
+  res->sum_r_payload = g[1];
+  res->sum_s_payload = g[2];
+  res->pair_checksum = g[3];
+  res->n_required = r[0];
+  res->n_written = mat ? std::min<uint64_t>(r[4], out->capacity) : 0;
+  res->n_items = (uint32_t)(r[5] & 0xFFFFFFFFu);
+  res->r_local = loc[0].n;
+  res->s_local = loc[1].n;
+  res->passes = pl.passes;
+  res->bits[0] = pl.bits[0];
+  res->bits[1] = pl.passes == 2 ? pl.bits[1] : 0;
+  res->n_partitions = Q;
+  if (mat && out->mem == HAPE_MEM_HOST && res->n_written) {
+    CK(h, cudaMemcpyAsync(out->r_payload, mat_r, res->n_written * prw, cudaMemcpyDeviceToHost, h->stream));
+    CK(h, cudaMemcpyAsync(out->s_payload, mat_s, res->n_written * psw, cudaMemcpyDeviceToHost, h->stream));
+  }
+  cudaEventRecord(h->ev[HAPE_NSTAGES], h->stream);
+  CK(h, cudaStreamSynchronize(h->stream));
+  res->kernel_launches = h->launches;
+  // stage times: each used stage runs until the next used stage mark
+  int order[HAPE_NSTAGES];
+  int no = 0;
+  for (int s = HAPE_STAGE_H2D; s < HAPE_STAGE_TOTAL; s++)
+    if (h->ev_used[s]) order[no++] = s;
+  for (int i = 0; i < no; i++) {
+    cudaEvent_t end = i + 1 < no ? h->ev[order[i + 1]] : h->ev[HAPE_NSTAGES];
+    float ms = 0;
+    cudaEventElapsedTime(&ms, h->ev[order[i]], end);
+    res->stage_ms[order[i]] = ms;
+  }
+  float tot = 0;
+  cudaEventElapsedTime(&tot, h->ev[HAPE_STAGE_TOTAL], h->ev[HAPE_NSTAGES]);
+  res->stage_ms[HAPE_STAGE_TOTAL] = tot;
+  (void)cudaGetLastError();
+  if (mat && r[4] > out->capacity)
+    return fail(h, HAPE_ERR_OUTPUT_CAPACITY, "join produced %llu pairs > capacity %llu", (unsigned long long)r[4],
+                (unsigned long long)out->capacity);
+  return HAPE_OK;
+}
+
+// ---------------------------------------------------------------------------
+// exported ABI
+// ---------------------------------------------------------------------------
+extern "C" {
+
+const char* hape_version(void) { return "hape-b200 1.0 (sm_100a, ABI 1)"; }
+
+const char* hape_status_string(hape_status s) {
+  switch (s) {
+    case HAPE_OK: return "HAPE_OK";
+    case HAPE_ERR_INVALID_ARG: return "HAPE_ERR_INVALID_ARG";
+    case HAPE_ERR_CUDA: return "HAPE_ERR_CUDA";
+    case HAPE_ERR_OOM: return "HAPE_ERR_OOM";
+    case HAPE_ERR_OUTPUT_CAPACITY: return "HAPE_ERR_OUTPUT_CAPACITY";
+    case HAPE_ERR_NCCL: return "HAPE_ERR_NCCL";
+    case HAPE_ERR_UNSUPPORTED: return "HAPE_ERR_UNSUPPORTED";
+  }
+  return "HAPE_ERR_UNKNOWN";
+}
+
+hape_status hape_join_create(const hape_join_config* cfg, hape_join** out_handle) {
+  if (!cfg || !out_handle) return HAPE_ERR_INVALID_ARG;
+  *out_handle = nullptr;
+  if (cfg->key_type != HAPE_INT32 && cfg->key_type != HAPE_INT64) return HAPE_ERR_INVALID_ARG;
+  if ((cfg->r_payload_type != HAPE_INT32 && cfg->r_payload_type != HAPE_INT64) ||
+      (cfg->s_payload_type != HAPE_INT32 && cfg->s_payload_type != HAPE_INT64))
+    return HAPE_ERR_INVALID_ARG;
+  if (cfg->part_fn != HAPE_PART_HASH && cfg->part_fn != HAPE_PART_IDENTITY) return HAPE_ERR_INVALID_ARG;
+  if (cfg->radix_passes < 0 || cfg->radix_passes > 2) return HAPE_ERR_INVALID_ARG;
+  if (cfg->radix_bits[0] < 0 || cfg->radix_bits[1] < 0 || cfg->radix_bits[0] > (int)kMaxBitsPerPass ||
+      cfg->radix_bits[1] > (int)kMaxBitsPerPass)
+    return HAPE_ERR_INVALID_ARG;
+  const int world = cfg->world_size > 1 ? cfg->world_size : 1;
+  if (cfg->world_size < 0 || (world & (world - 1)) != 0) return HAPE_ERR_INVALID_ARG;
+  if (cfg->rank < 0 || cfg->rank >= world) return HAPE_ERR_INVALID_ARG;
+  if (world > 1 && !cfg->nccl_comm) return HAPE_ERR_INVALID_ARG;
+  if (cfg->device < 0) return HAPE_ERR_INVALID_ARG;
+  int ndev = 0;
+  if (cudaGetDeviceCount(&ndev) != cudaSuccess || cfg->device >= ndev) {
+    (void)cudaGetLastError();
+    return HAPE_ERR_CUDA;
+  }
+  hape_join* h = new hape_join();
+  h->cfg = *cfg;
+  h->dev = cfg->device;
+  h->comm = static_cast<ncclComm_t>(cfg->nccl_comm);
+  hape_status st = HAPE_OK;
+  do {
+    if (cudaSetDevice(h->dev) != cudaSuccess) { st = HAPE_ERR_CUDA; break; }
+    cudaDeviceGetAttribute(&h->num_sms, cudaDevAttrMultiProcessorCount, h->dev);
+    if (cfg->stream) {
+      h->stream = static_cast<cudaStream_t>(cfg->stream);
+    } else {
+      if (cudaStreamCreateWithFlags(&h->stream, cudaStreamNonBlocking) != cudaSuccess) { st = HAPE_ERR_CUDA; break; }
+      h->own_stream = true;
+    }
+    for (auto& e : h->ev)
+      if (cudaEventCreate(&e) != cudaSuccess) { st = HAPE_ERR_CUDA; break; }
+    if (st != HAPE_OK) break;
+    if (cudaMallocHost(&h->h_res, 16 * sizeof(unsigned long long)) != cudaSuccess) { st = HAPE_ERR_OOM; break; }
+    if (cfg->max_r || cfg->max_s) {
+      hape_plan pl;
+      if (make_plan(h, cfg->max_r, cfg->max_s, &pl) == HAPE_OK) {
+        const CallLayout L = layout_for(h, pl, cfg->max_r, cfg->max_s);
+        if (ensure(h, h->small, L.total) != HAPE_OK) { st = HAPE_ERR_OOM; break; }
+      }
+    }
+  } while (0);
+  if (st != HAPE_OK) {
+    (void)cudaGetLastError();
+    hape_join_destroy(h);
+    return st;
+  }
+  *out_handle = h;
+  return HAPE_OK;
+}
+
+hape_status hape_join_destroy(hape_join* h) {
+  if (!h) return HAPE_OK;
+  cudaSetDevice(h->dev);
+  if (h->stream) cudaStreamSynchronize(h->stream);
+  DevBuf* groups[] = {h->stage, h->ping, h->pong, h->send, h->recv};
+  for (DevBuf* g : groups)
+    for (int i = 0; i < 4; i++)
+      if (g[i].p) cudaFree(g[i].p);
+  for (auto& b : h->outst)
+    if (b.p) cudaFree(b.p);
+  if (h->small.p) cudaFree(h->small.p);
+  if (h->h_res) cudaFreeHost(h->h_res);
+  if (h->h_bounds) cudaFreeHost(h->h_bounds);
+  for (auto& e : h->ev)
+    if (e) cudaEventDestroy(e);
+  if (h->own_stream && h->stream) cudaStreamDestroy(h->stream);
+  (void)cudaGetLastError();
+  delete h;
+  return HAPE_OK;
+}
+
+const char* hape_last_error(const hape_join* h) { return h ? h->err.c_str() : "NULL handle"; }
+
+hape_status hape_join_plan(const hape_join* h, uint64_t n_r, uint64_t n_s, hape_plan* out) {
+  if (!h || !out) return HAPE_ERR_INVALID_ARG;
+  return make_plan(h, n_r, n_s, out);
+}
+
+hape_status hape_radix_join(hape_join* h, const hape_relation* R, const hape_relation* S, const hape_output* out,
+                            hape_join_result* res) {
+  if (!h) return HAPE_ERR_INVALID_ARG;
+  if (!res) return fail(h, HAPE_ERR_INVALID_ARG, "res is NULL");
+  try {
+    return join_impl(h, R, S, out, res);
+  } catch (...) {
+    return fail(h, HAPE_ERR_CUDA, "unexpected C++ exception");
+  }
+}
+
+hape_status hape_debug_partition(hape_join* h, const hape_relation* rel, int is_s, const hape_plan* plan_in,
+                                 void* out_keys, void* out_payloads, uint32_t* out_bounds, hape_plan* plan_out) {
+  if (!h) return HAPE_ERR_INVALID_ARG;
+  const hape_join_config& c = h->cfg;
+  const int kw = key_width(c), pw = pay_width(is_s ? c.s_payload_type : c.r_payload_type);
+  CKS(check_rel(h, rel, kw, pw, "rel"));
+  if (rel->n && (!out_keys || !out_payloads)) return fail(h, HAPE_ERR_INVALID_ARG, "outputs NULL");
+  if (!out_bounds) return fail(h, HAPE_ERR_INVALID_ARG, "out_bounds NULL");
+  CK(h, cudaSetDevice(h->dev));
+  hape_plan pl;
+  if (plan_in) pl = *plan_in;
+  else if (make_plan(h, rel->n, rel->n, &pl) != HAPE_OK) return fail(h, HAPE_ERR_INVALID_ARG, "invalid plan");
+  if (pl.passes < 1 || pl.passes > 2 || pl.bits[0] > kMaxBitsPerPass || pl.bits[1] > kMaxBitsPerPass)
+    return fail(h, HAPE_ERR_INVALID_ARG, "invalid plan");
+  h->launches = 0;
+  Col in;
+  CKS(stage_in(h, rel, kw, pw, h->stage[0], h->stage[1], &in));
+  const CallLayout L = layout_for(h, pl, rel->n, rel->n);
+  CKS(ensure(h, h->small, L.total));
+  CKS(ensure(h, h->ping[0], rel->n * kw + 16));
+  CKS(ensure(h, h->ping[1], rel->n * pw + 16));
+  CKS(ensure(h, h->pong[0], rel->n * kw + 16));
+  CKS(ensure(h, h->pong[1], rel->n * pw + 16));
+  CK(h, cudaMemsetAsync(at<char>(h, L.zero_lo), 0, L.zero_hi - L.zero_lo, h->stream));
+  PassIO io[2];
+  io[0] = PassIO{in, h->ping[0].p, h->ping[1].p, h->pong[0].p, h->pong[1].p};
+  const void* fk[2];
+  const void* fp[2];
+  const uint32_t* fb[2];
+  CKS(run_partition_stages(h, pl, L, io, 1, fk, fp, fb));
+  const uint64_t Q = 1ull << (pl.bits[0] + (pl.passes == 2 ? pl.bits[1] : 0));
+  if (rel->n) {
+    CK(h, cudaMemcpyAsync(out_keys, fk[0], rel->n * kw, cudaMemcpyDeviceToDevice, h->stream));
+    CK(h, cudaMemcpyAsync(out_payloads, fp[0], rel->n * pw, cudaMemcpyDeviceToDevice, h->stream));
+  }
+  CK(h, cudaMemcpyAsync(out_bounds, fb[0], (Q + 1) * 4, cudaMemcpyDeviceToDevice, h->stream));
+  CK(h, cudaStreamSynchronize(h->stream));
+  if (plan_out) *plan_out = pl;
+  return HAPE_OK;
+}
+
+hape_status hape_nccl_unique_id(void* out_id_128) {
+  if (!out_id_128) return HAPE_ERR_INVALID_ARG;
+  static_assert(sizeof(ncclUniqueId) == 128, "ncclUniqueId size");
+  ncclUniqueId id;
+  if (ncclGetUniqueId(&id) != ncclSuccess) return HAPE_ERR_NCCL;
+  memcpy(out_id_128, &id, sizeof id);
+  return HAPE_OK;
+}
+
+hape_status hape_nccl_comm_init(const void* id_128, int world_size, int rank, int device, void** out_comm) {
+  if (!id_128 || !out_comm || world_size < 1 || rank < 0 || rank >= world_size) return HAPE_ERR_INVALID_ARG;
+  if (cudaSetDevice(device) != cudaSuccess) { (void)cudaGetLastError(); return HAPE_ERR_CUDA; }
+  ncclUniqueId id;
+  memcpy(&id, id_128, sizeof id);
+  ncclComm_t comm;
+  if (ncclCommInitRank(&comm, world_size, id, rank) != ncclSuccess) return HAPE_ERR_NCCL;
+  *out_comm = comm;
+  return HAPE_OK;
+}
+
+hape_status hape_nccl_comm_destroy(void* comm) {
+  if (!comm) return HAPE_OK;
+  return ncclCommDestroy(static_cast<ncclComm_t>(comm)) == ncclSuccess ? HAPE_OK : HAPE_ERR_NCCL;
+}
+
+}  // extern "C"

@@ -1,0 +1,520 @@
+// kernels.cuh -- sm_100a kernels of the partitioned radix hash equi-join.
+//
+// PAPER.md §4.1 (P528-598, Figs. 3-4) is the method:
+//   * a partitioning pass reads "a chunk of the input (at a time) in the
+//     scratchpad and reorganize[s] it in such a way that elements belonging
+//     to the same output partition are located in consecutive scratchpad
+//     entries. Then, we scan the scratchpad and write each tuple to its
+//     corresponding output partition" (P579-584)  -> k_scatter;
+//   * its write offsets come from histogram + exclusive scan, the two-scan
+//     method of [27] that BASELINE.json's north_star mandates (the paper
+//     contrasts it with its linked buffers, P593-597)  -> k_hist, k_scan;
+//   * fan-out is bounded by the scratchpad that consolidates the stores, so
+//     the join runs 1-2 passes (P531-534, P589-593);
+//   * per co-partition: "load the smaller partition to the scratchpad, build
+//     the hash-table using atomic operations and probe with the tuples of the
+//     corresponding partition" (P537-540)  -> k_build_probe;
+//   * the micro-benchmark consumer: count and sum over each payload column
+//     (P789-793), fused into the probe epilogue.
+//
+// Data layout in HBM: structure-of-arrays everywhere (caller columns and the
+// ping-pong workspace), uint32 tuple indices (n < 2^32 per relation per rank).
+// Nothing here is a dense contraction: no tensor cores.
+#pragma once
+#include <cstdint>
+#include <cuda_runtime.h>
+
+namespace hape {
+
+// --------------------------------------------------------------------------
+// widths and the partition function (reading R1)
+// --------------------------------------------------------------------------
+template <int W> struct UW;
+template <> struct UW<4> { using T = uint32_t; using S = int32_t; };
+template <> struct UW<8> { using T = uint64_t; using S = int64_t; };
+
+__device__ __forceinline__ uint32_t fmix32(uint32_t h) {
+  h ^= h >> 16; h *= 0x85ebca6bu;
+  h ^= h >> 13; h *= 0xc2b2ae35u;
+  h ^= h >> 16;
+  return h;
+}
+
+__device__ __forceinline__ uint64_t fmix64(uint64_t x) {
+  x ^= x >> 30; x *= 0xbf58476d1ce4e5b9ull;
+  x ^= x >> 27; x *= 0x94d049bb133111ebull;
+  x ^= x >> 31;
+  return x;
+}
+
+// h(k): bijective mixer of the key bit pattern, or identity (P802-804)
+template <int KW>
+__device__ __forceinline__ uint64_t part_hash(typename UW<KW>::T k, int ident) {
+  if (ident) return (uint64_t)k;
+  if constexpr (KW == 4) return (uint64_t)fmix32(k);
+  else return fmix64(k);
+}
+
+// bucket = (h >> shift) & mask  (R3: dest = top bits, pass k = low bits)
+struct BitField { uint32_t shift; uint32_t mask; };
+
+__device__ __forceinline__ uint32_t bucket_of(uint64_t h, BitField bf) {
+  return (uint32_t)(h >> bf.shift) & bf.mask;
+}
+
+// pair-checksum term (R10): mix(p,q) = fmix64(p*phi + fmix64(q))
+__device__ __forceinline__ uint64_t pair_mix(int64_t p, int64_t q) {
+  return fmix64((uint64_t)p * 0x9E3779B97F4A7C15ull + fmix64((uint64_t)q));
+}
+
+// --------------------------------------------------------------------------
+// segment -> CTA chunk mapping, shared by k_hist and k_scatter of one pass
+// (the offsets are only right if both kernels see identical chunks)
+// --------------------------------------------------------------------------
+struct SegMap {
+  const uint32_t* bounds;  // nseg+1 segment bounds (device) or nullptr: one segment [0, n)
+  uint32_t nseg;
+  uint32_t cps;            // CTAs per segment
+  uint32_t n;
+};
+
+__device__ __forceinline__ void seg_chunk(const SegMap& m, uint32_t cta, uint32_t& seg,
+                                          uint32_t& j, uint32_t& lo, uint32_t& hi) {
+  seg = cta / m.cps;
+  j = cta - seg * m.cps;
+  uint32_t b = m.bounds ? m.bounds[seg] : 0u;
+  uint32_t e = m.bounds ? m.bounds[seg + 1] : m.n;
+  uint64_t len = (uint64_t)(e - b);
+  lo = b + (uint32_t)((len * j) / m.cps);
+  hi = b + (uint32_t)((len * (j + 1)) / m.cps);
+}
+
+// --------------------------------------------------------------------------
+// small block primitives
+// --------------------------------------------------------------------------
+__device__ __forceinline__ uint32_t warp_incl_scan(uint32_t v) {
+  const int lane = threadIdx.x & 31;
+#pragma unroll
+  for (int o = 1; o < 32; o <<= 1) {
+    uint32_t t = __shfl_up_sync(0xffffffffu, v, o);
+    if (lane >= o) v += t;
+  }
+  return v;
+}
+
+// In-place exclusive scan of a[0..n) in shared memory; returns the total.
+// All threads of the block must call it.  wtmp: >= 33 words of smem.
+template <int BD>
+__device__ uint32_t block_exscan_smem(uint32_t* a, int n, uint32_t* wtmp) {
+  const int tid = threadIdx.x, lane = tid & 31, warp = tid >> 5;
+  constexpr int NW = BD / 32;
+  const int c = (n + BD - 1) / BD;
+  const int lo = min(tid * c, n), hi = min(lo + c, n);
+  uint32_t s = 0;
+  for (int i = lo; i < hi; i++) s += a[i];
+  uint32_t incl = warp_incl_scan(s);
+  if (lane == 31) wtmp[warp] = incl;
+  __syncthreads();
+  if (warp == 0) {
+    uint32_t v = lane < NW ? wtmp[lane] : 0u;
+    uint32_t vi = warp_incl_scan(v);
+    if (lane < NW) wtmp[lane] = vi - v;
+    if (lane == 31) wtmp[32] = vi;
+  }
+  __syncthreads();
+  uint32_t ex = wtmp[warp] + incl - s;
+  for (int i = lo; i < hi; i++) { uint32_t t = a[i]; a[i] = ex; ex += t; }
+  uint32_t total = wtmp[32];
+  __syncthreads();
+  return total;
+}
+
+// --------------------------------------------------------------------------
+// a6: radix histogram of one pass.  One contiguous chunk per CTA; keys only
+// (w_k bytes per tuple); shared-memory counters (P166-168: "use shared memory
+// to store histograms").  Output hist[(seg*P + p)*cps + j] (partition-major
+// inside each segment, so the segment's exclusive scan IS the offsets) and
+// the per-row totals rowsum[seg*P + p].
+// --------------------------------------------------------------------------
+constexpr int HIST_THREADS = 512;
+
+template <int KW>
+__global__ void __launch_bounds__(HIST_THREADS)
+k_hist(const typename UW<KW>::T* __restrict__ key, SegMap m, BitField bf, int ident, uint32_t P,
+       uint32_t* __restrict__ hist, uint32_t* __restrict__ rowsum) {
+  extern __shared__ uint32_t sh_cnt[];
+  using K = typename UW<KW>::T;
+  for (uint32_t i = threadIdx.x; i < P; i += HIST_THREADS) sh_cnt[i] = 0;
+  __syncthreads();
+  uint32_t seg, j, lo, hi;
+  seg_chunk(m, blockIdx.x, seg, j, lo, hi);
+  constexpr int U = 4;
+  uint32_t i = lo + threadIdx.x;
+  for (; i + (U - 1) * HIST_THREADS < hi; i += U * HIST_THREADS) {
+    K k[U];
+#pragma unroll
+    for (int u = 0; u < U; u++) k[u] = __ldcs(key + i + u * HIST_THREADS);
+#pragma unroll
+    for (int u = 0; u < U; u++) atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(k[u], ident), bf)], 1u);
+  }
+  for (; i < hi; i += HIST_THREADS) atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(__ldcs(key + i), ident), bf)], 1u);
+  __syncthreads();
+  const uint32_t row0 = seg * P;
+  for (uint32_t p = threadIdx.x; p < P; p += HIST_THREADS) {
+    uint32_t c = sh_cnt[p];
+    hist[(size_t)(row0 + p) * m.cps + j] = c;
+    if (c) atomicAdd(&rowsum[row0 + p], c);
+  }
+}
+
+// --------------------------------------------------------------------------
+// a7: exclusive prefix sum of the histograms -> absolute write offsets (in
+// place) and the partition bounds of the pass.  CTA (seg, row-group) scans a
+// contiguous tile of rows; the tile's base is the segment start plus the sum
+// of earlier rows' totals (rowsum), so no inter-CTA waiting is needed.
+// --------------------------------------------------------------------------
+constexpr int SCAN_THREADS = 256;
+constexpr int SCAN_TILE = 4096;
+
+__global__ void __launch_bounds__(SCAN_THREADS)
+k_scan(uint32_t* __restrict__ hist, const uint32_t* __restrict__ rowsum, SegMap m, uint32_t P,
+       uint32_t rows_per_cta, uint32_t* __restrict__ bounds_out) {
+  __shared__ uint32_t tile[SCAN_TILE];
+  __shared__ uint32_t wtmp[33];
+  __shared__ uint32_t s_prefix;
+  const uint32_t groups = (P + rows_per_cta - 1) / rows_per_cta;
+  const uint32_t seg = blockIdx.x / groups, g = blockIdx.x - seg * groups;
+  const uint32_t p0 = g * rows_per_cta, p1 = min(P, p0 + rows_per_cta);
+  const uint32_t row0 = seg * P;
+  // prefix = sum of rowsum over rows [0, p0) of this segment
+  uint32_t s = 0;
+  for (uint32_t p = threadIdx.x; p < p0; p += SCAN_THREADS) s += rowsum[row0 + p];
+  for (int o = 16; o > 0; o >>= 1) s += __shfl_xor_sync(0xffffffffu, s, o);
+  if (threadIdx.x == 0) s_prefix = 0;
+  __syncthreads();
+  if ((threadIdx.x & 31) == 0 && s) atomicAdd(&s_prefix, s);
+  __syncthreads();
+  const uint32_t seg_base = m.bounds ? m.bounds[seg] : 0u;
+  uint32_t carry = seg_base + s_prefix;
+  const size_t e0 = (size_t)(row0 + p0) * m.cps, e1 = (size_t)(row0 + p1) * m.cps;
+  for (size_t c0 = e0; c0 < e1; c0 += SCAN_TILE) {
+    const int cn = (int)min((size_t)SCAN_TILE, e1 - c0);
+    for (int i = threadIdx.x; i < cn; i += SCAN_THREADS) tile[i] = hist[c0 + i];
+    __syncthreads();
+    uint32_t tot = block_exscan_smem<SCAN_THREADS>(tile, cn, wtmp);
+    for (int i = threadIdx.x; i < cn; i += SCAN_THREADS) {
+      uint32_t off = carry + tile[i];
+      hist[c0 + i] = off;
+      size_t e = c0 + i;
+      if (e % m.cps == 0) bounds_out[e / m.cps] = off;  // row start = partition bound
+    }
+    carry += tot;
+    __syncthreads();
+  }
+  if (seg == m.nseg - 1 && g == groups - 1 && threadIdx.x == 0)
+    bounds_out[(size_t)m.nseg * P] = m.bounds ? m.bounds[m.nseg] : m.n;
+}
+
+// --------------------------------------------------------------------------
+// a8/a9: smem-staged, write-combined scatter (Fig. 4, P579-589).
+// Per tile of SC_TILE tuples: load (coalesced), compute the bucket, claim a
+// rank with a shared-memory atomic, exclusive-scan the tile's bucket counts,
+// reorder the tile in shared memory so each bucket is a consecutive run, then
+// write the runs with consecutive threads -> consecutive addresses (the runs
+// of one bucket continue where the previous tile's stopped, so L2 merges
+// partial sectors before they reach HBM).
+// --------------------------------------------------------------------------
+constexpr int SC_THREADS = 512;
+constexpr int SC_ITEMS = 8;
+constexpr int SC_TILE = SC_THREADS * SC_ITEMS;
+
+template <int KW, int PW>
+__host__ __device__ constexpr size_t scatter_smem_bytes(uint32_t P) {
+  return (size_t)SC_TILE * (KW + PW + 2) + (size_t)P * 12 + 33 * 4;
+}
+
+template <int KW, int PW>
+__global__ void __launch_bounds__(SC_THREADS, 2)
+k_scatter(const typename UW<KW>::T* __restrict__ ik, const typename UW<PW>::T* __restrict__ ip,
+          SegMap m, BitField bf, int ident, uint32_t P, const uint32_t* __restrict__ offsets,
+          typename UW<KW>::T* __restrict__ ok, typename UW<PW>::T* __restrict__ op) {
+  using K = typename UW<KW>::T;
+  using V = typename UW<PW>::T;
+  extern __shared__ __align__(16) unsigned char smem[];
+  K* s_key = reinterpret_cast<K*>(smem);
+  V* s_pay = reinterpret_cast<V*>(smem + (size_t)SC_TILE * KW);
+  uint16_t* s_bkt = reinterpret_cast<uint16_t*>(smem + (size_t)SC_TILE * (KW + PW));
+  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(smem + (size_t)SC_TILE * (KW + PW + 2));
+  uint32_t* s_cur = s_cnt + P;     // running absolute write cursor per bucket
+  uint32_t* s_dlt = s_cur + P;     // cursor - tile start of the bucket
+  uint32_t* wtmp = s_dlt + P;
+
+  uint32_t seg, j, lo, hi;
+  seg_chunk(m, blockIdx.x, seg, j, lo, hi);
+  const uint32_t row0 = seg * P;
+  for (uint32_t p = threadIdx.x; p < P; p += SC_THREADS)
+    s_cur[p] = offsets[(size_t)(row0 + p) * m.cps + j];
+
+  for (uint32_t t0 = lo; t0 < hi; t0 += SC_TILE) {
+    const uint32_t tn = min((uint32_t)SC_TILE, hi - t0);
+    for (uint32_t p = threadIdx.x; p < P; p += SC_THREADS) s_cnt[p] = 0;
+    __syncthreads();
+    K k[SC_ITEMS];
+    V v[SC_ITEMS];
+    uint32_t b[SC_ITEMS], r[SC_ITEMS];
+#pragma unroll
+    for (int u = 0; u < SC_ITEMS; u++) {
+      const uint32_t i = u * SC_THREADS + threadIdx.x;
+      if (i < tn) { k[u] = __ldcs(ik + t0 + i); v[u] = __ldcs(ip + t0 + i); }
+    }
+#pragma unroll
+    for (int u = 0; u < SC_ITEMS; u++) {
+      const uint32_t i = u * SC_THREADS + threadIdx.x;
+      if (i < tn) {
+        b[u] = bucket_of(part_hash<KW>(k[u], ident), bf);
+        r[u] = atomicAdd(&s_cnt[b[u]], 1u);
+      }
+    }
+    __syncthreads();
+    // tile start of every bucket; delta = where the bucket's run goes in HBM
+    // minus where it sits in the reordered tile
+    for (uint32_t p = threadIdx.x; p < P; p += SC_THREADS) s_dlt[p] = s_cnt[p];
+    __syncthreads();
+    block_exscan_smem<SC_THREADS>(s_dlt, (int)P, wtmp);  // s_dlt = tile start
+    for (uint32_t p = threadIdx.x; p < P; p += SC_THREADS) {
+      const uint32_t st = s_dlt[p], c = s_cnt[p], cur = s_cur[p];
+      s_dlt[p] = cur - st;
+      s_cnt[p] = st;                                     // keep the start for placement
+      s_cur[p] = cur + c;
+    }
+    __syncthreads();
+#pragma unroll
+    for (int u = 0; u < SC_ITEMS; u++) {
+      const uint32_t i = u * SC_THREADS + threadIdx.x;
+      if (i < tn) {
+        const uint32_t pos = s_cnt[b[u]] + r[u];
+        s_key[pos] = k[u];
+        s_pay[pos] = v[u];
+        s_bkt[pos] = (uint16_t)b[u];
+      }
+    }
+    __syncthreads();
+    for (uint32_t i = threadIdx.x; i < tn; i += SC_THREADS) {
+      const uint32_t dst = s_dlt[s_bkt[i]] + i;
+      ok[dst] = s_key[i];
+      op[dst] = s_pay[i];
+    }
+    __syncthreads();
+  }
+}
+
+// --------------------------------------------------------------------------
+// a10: co-partition work list.  Item = (partition q, S-slice index); one item
+// per probe_slice S tuples of a non-empty co-partition (skewed S partitions
+// are split across CTAs; R partitions larger than the smem build capacity
+// are chunked inside the item).  Zip of co-partitions, P740-747; one
+// co-partition per thread block, P804-806.
+// --------------------------------------------------------------------------
+constexpr int WL_THREADS = 1024;
+
+__global__ void __launch_bounds__(WL_THREADS)
+k_worklist(const uint32_t* __restrict__ bR, const uint32_t* __restrict__ bS, uint32_t Q,
+           uint32_t slice, uint2* __restrict__ items, uint32_t* __restrict__ n_items) {
+  __shared__ uint32_t sc[WL_THREADS];
+  __shared__ uint32_t wtmp[33];
+  __shared__ uint32_t s_base;
+  const uint32_t q = blockIdx.x * WL_THREADS + threadIdx.x;
+  uint32_t k = 0;
+  if (q < Q) {
+    const uint32_t nr = bR[q + 1] - bR[q], ns = bS[q + 1] - bS[q];
+    k = (nr && ns) ? (ns + slice - 1) / slice : 0u;
+  }
+  sc[threadIdx.x] = k;
+  __syncthreads();
+  const uint32_t tot = block_exscan_smem<WL_THREADS>(sc, WL_THREADS, wtmp);
+  if (threadIdx.x == 0) s_base = tot ? atomicAdd(n_items, tot) : 0u;
+  __syncthreads();
+  const uint32_t base = s_base + sc[threadIdx.x];
+  for (uint32_t t = 0; t < k; t++) items[base + t] = make_uint2(q, t);
+}
+
+// --------------------------------------------------------------------------
+// a11-a13: per-co-partition build + probe with the hash table in shared
+// memory (Fig. 3, P535-541, P806-810), aggregation fused (P789-793),
+// optional materialisation through a block-aggregated output claim
+// ("Buffer output ... ATOMICS!", Fig. 3 P488-493).
+//
+// Persistent CTAs pull items from an atomic counter.  Shared memory holds the
+// R chunk (keys, payloads), next[] chain links (u16) and epoch-tagged chain
+// heads[2^slot_bits] (u32: epoch<<16 | index), so no head reset is needed
+// between builds.  The slot uses hash bits above the radix bits (every tuple
+// of a co-partition shares those).
+// --------------------------------------------------------------------------
+constexpr int JN_THREADS = 256;
+constexpr int JN_U = 4;
+constexpr uint32_t JN_NIL = 0xFFFFu;
+
+template <int KW, int PRW, int PSW>
+__host__ __device__ constexpr size_t join_smem_bytes(uint32_t cap, uint32_t slot_bits) {
+  return (size_t)cap * (KW + PRW) + (size_t)cap * 2 + ((size_t)4 << slot_bits) + 16;
+}
+
+struct JoinArgs {
+  const void* rk; const void* rp; const void* sk; const void* sp;
+  const uint32_t* bR; const uint32_t* bS;
+  const uint2* items; const uint32_t* n_items; uint32_t* item_ctr;
+  uint32_t cap; uint32_t slice; uint32_t slot_shift; uint32_t slot_bits; int ident;
+  unsigned long long* acc;       // [4] count, sum_r, sum_s, checksum
+  void* out_r; void* out_s; unsigned long long out_cap; unsigned long long* out_ctr;
+};
+
+template <int KW, int PRW, int PSW, bool MAT>
+__global__ void __launch_bounds__(JN_THREADS)
+k_build_probe(JoinArgs a) {
+  using K = typename UW<KW>::T;
+  using PR = typename UW<PRW>::S;
+  using PS = typename UW<PSW>::S;
+  extern __shared__ __align__(16) unsigned char smem[];
+  K* s_rk = reinterpret_cast<K*>(smem);
+  PR* s_rp = reinterpret_cast<PR*>(smem + (size_t)a.cap * KW);
+  uint16_t* s_next = reinterpret_cast<uint16_t*>(smem + (size_t)a.cap * (KW + PRW));
+  uint32_t* s_head = reinterpret_cast<uint32_t*>(smem + (size_t)a.cap * (KW + PRW + 2) +
+                                                  (((size_t)a.cap * 2) & 2));  // 4-B align
+  __shared__ uint32_t s_item;
+  __shared__ uint32_t s_wsum[JN_THREADS / 32];
+  __shared__ unsigned long long s_wbase[JN_THREADS / 32];
+  __shared__ unsigned long long s_red[4][JN_THREADS / 32];
+
+  const K* __restrict__ rk = static_cast<const K*>(a.rk);
+  const PR* __restrict__ rp = static_cast<const PR*>(a.rp);
+  const K* __restrict__ sk = static_cast<const K*>(a.sk);
+  const PS* __restrict__ sp = static_cast<const PS*>(a.sp);
+  const uint32_t nslots = 1u << a.slot_bits, smask = nslots - 1;
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+
+  unsigned long long cnt = 0, sr = 0, ss = 0, sx = 0;
+  uint32_t epoch = 0;  // heads with another epoch are empty
+  for (uint32_t i = threadIdx.x; i < nslots; i += JN_THREADS) s_head[i] = 0;
+  const uint32_t n_items = *a.n_items;
+
+  while (true) {
+    __syncthreads();
+    if (threadIdx.x == 0) s_item = atomicAdd(a.item_ctr, 1u);
+    __syncthreads();
+    const uint32_t it = s_item;
+    if (it >= n_items) break;
+    const uint2 item = a.items[it];
+    const uint32_t q = item.x;
+    const uint32_t r_lo = a.bR[q], r_hi = a.bR[q + 1];
+    const uint32_t s_lo = a.bS[q] + item.y * a.slice;
+    const uint32_t s_hi = min(a.bS[q + 1], s_lo + a.slice);
+
+    for (uint32_t c_lo = r_lo; c_lo < r_hi; c_lo += a.cap) {
+      const uint32_t nr = min(a.cap, r_hi - c_lo);
+      if (++epoch == 0x10000u) {  // epoch wrap: clear the heads once
+        for (uint32_t i = threadIdx.x; i < nslots; i += JN_THREADS) s_head[i] = 0;
+        epoch = 1;
+        __syncthreads();
+      }
+      // ---- build (a11): R chunk -> smem, chained table via atomicExch
+      for (uint32_t i = threadIdx.x; i < nr; i += JN_THREADS) {
+        const K k = rk[c_lo + i];
+        s_rk[i] = k;
+        s_rp[i] = rp[c_lo + i];
+        const uint32_t slot = (uint32_t)(part_hash<KW>(k, a.ident) >> a.slot_shift) & smask;
+        const uint32_t old = atomicExch(&s_head[slot], (epoch << 16) | i);
+        s_next[i] = (old >> 16) == epoch ? (uint16_t)(old & 0xFFFFu) : (uint16_t)JN_NIL;
+      }
+      __syncthreads();
+      // ---- probe (a12): stream the S slice
+      for (uint32_t base = s_lo; base < s_hi; base += JN_THREADS * JN_U) {
+        K k[JN_U];
+        PS v[JN_U];
+        uint32_t head[JN_U];
+#pragma unroll
+        for (int u = 0; u < JN_U; u++) {
+          const uint32_t j = base + u * JN_THREADS + threadIdx.x;
+          if (j < s_hi) { k[u] = __ldcs(sk + j); v[u] = __ldcs(sp + j); }
+        }
+#pragma unroll
+        for (int u = 0; u < JN_U; u++) {
+          const uint32_t j = base + u * JN_THREADS + threadIdx.x;
+          head[u] = JN_NIL;
+          if (j < s_hi) {
+            const uint32_t slot = (uint32_t)(part_hash<KW>(k[u], a.ident) >> a.slot_shift) & smask;
+            const uint32_t h = s_head[slot];
+            head[u] = (h >> 16) == epoch ? (h & 0xFFFFu) : JN_NIL;
+          }
+        }
+        uint32_t c[JN_U];
+#pragma unroll
+        for (int u = 0; u < JN_U; u++) {
+          c[u] = 0;
+          for (uint32_t e = head[u]; e != JN_NIL; e = s_next[e]) {
+            if (s_rk[e] == k[u]) {
+              const int64_t pr = (int64_t)s_rp[e], ps = (int64_t)v[u];
+              c[u]++;
+              sr += (unsigned long long)pr;
+              ss += (unsigned long long)ps;
+              sx += pair_mix(pr, ps);
+            }
+          }
+          cnt += c[u];
+        }
+        if constexpr (MAT) {
+          // positions: (u-major, lane-minor) order inside the warp, warps in
+          // order inside the block, one global claim per block per batch
+          uint32_t incl[JN_U], wtot = 0, before[JN_U];
+#pragma unroll
+          for (int u = 0; u < JN_U; u++) {
+            incl[u] = warp_incl_scan(c[u]);
+            before[u] = wtot;
+            wtot += __shfl_sync(0xffffffffu, incl[u], 31);
+          }
+          if (lane == 0) s_wsum[warp] = wtot;
+          __syncthreads();
+          if (threadIdx.x == 0) {
+            unsigned long long run = 0;
+            for (int w = 0; w < JN_THREADS / 32; w++) { s_wbase[w] = run; run += s_wsum[w]; }
+            const unsigned long long g = run ? atomicAdd(a.out_ctr, run) : 0ull;
+            for (int w = 0; w < JN_THREADS / 32; w++) s_wbase[w] += g;
+          }
+          __syncthreads();
+          const unsigned long long wb = s_wbase[warp];
+#pragma unroll
+          for (int u = 0; u < JN_U; u++) {
+            if (!c[u]) continue;
+            unsigned long long pos = wb + before[u] + incl[u] - c[u];
+            for (uint32_t e = head[u]; e != JN_NIL; e = s_next[e]) {
+              if (s_rk[e] == k[u]) {
+                if (pos < a.out_cap) {
+                  static_cast<PR*>(a.out_r)[pos] = s_rp[e];
+                  static_cast<PS*>(a.out_s)[pos] = v[u];
+                }
+                pos++;
+              }
+            }
+          }
+        }
+      }
+      __syncthreads();
+    }
+  }
+  // ---- a13: block reduction of the four u64 partials, one atomic each
+#pragma unroll
+  for (int o = 16; o > 0; o >>= 1) {
+    cnt += __shfl_xor_sync(0xffffffffu, cnt, o);
+    sr += __shfl_xor_sync(0xffffffffu, sr, o);
+    ss += __shfl_xor_sync(0xffffffffu, ss, o);
+    sx += __shfl_xor_sync(0xffffffffu, sx, o);
+  }
+  if (lane == 0) { s_red[0][warp] = cnt; s_red[1][warp] = sr; s_red[2][warp] = ss; s_red[3][warp] = sx; }
+  __syncthreads();
+  if (threadIdx.x < 4) {
+    unsigned long long t = 0;
+    for (int w = 0; w < JN_THREADS / 32; w++) t += s_red[threadIdx.x][w];
+    if (t) atomicAdd(&a.acc[threadIdx.x], t);
+  }
+}
+
+}  // namespace hape

@@ -1,0 +1,252 @@
+"""GPU parity: the CUDA path (through the C ABI) vs the CPU oracle, element by
+element on the same seeded inputs.  All results are integers, so the bar is
+bit-exact: count, sum_r, sum_s, pair_checksum, and the sorted pair multiset.
+"""
+import numpy as np
+import pytest
+import torch
+
+import datagen
+import oracle
+from oracle import partition, provenance
+
+pytestmark = pytest.mark.gpu
+
+if torch.cuda.is_available():
+    from paper_conf_cidr_chrysogelossa19_b200 import HapeError, RadixJoin, _lib
+
+M64 = (1 << 64) - 1
+DT = {32: torch.int32, 64: torch.int64}
+
+
+def cuda(a):
+    return torch.as_tensor(np.ascontiguousarray(a)).cuda()
+
+
+def oracle_res(rk, rp, sk, sp, materialize=False):
+    return oracle.join(rk, rp, sk, sp, materialize=materialize)
+
+
+def check(res, want):
+    got = dict(count=res.match_count, sum_r=res.sum_r_payload, sum_s=res.sum_s_payload,
+               checksum=res.pair_checksum)
+    assert got == {k: want[k] for k in got}, (got, want)
+
+
+def sorted_pairs(a, b):
+    a = a.cpu().numpy().astype(np.int64)
+    b = b.cpu().numpy().astype(np.int64)
+    o = np.lexsort((b, a))
+    return a[o], b[o]
+
+
+_handles = {}
+
+
+def joiner(kdt, rdt=None, sdt=None, **kw):
+    key = (kdt, rdt, sdt, tuple(sorted(kw.items())))
+    if key not in _handles:
+        _handles[key] = RadixJoin(key_dtype=kdt, r_payload_dtype=rdt or kdt, s_payload_dtype=sdt or kdt, **kw)
+    return _handles[key]
+
+
+# --------------------------------------------------------------------------
+@pytest.mark.parametrize("seed", range(40))
+def test_random_small_vs_oracle(seed):
+    rng = np.random.default_rng(1000 + seed)
+    kb = [32, 64][seed % 2]
+    rb = [32, 64][(seed // 2) % 2]
+    sb = [32, 64][(seed // 4) % 2]
+    nr = int(rng.choice([0, 1, 5, 100, 4097, 20000, 70001]))
+    ns = int(rng.choice([0, 1, 7, 100, 4096, 30011, 65537]))
+    dom = int(rng.choice([1, 3, 64, 5000, 1 << 30]))
+    kdt = np.int32 if kb == 32 else np.int64
+    rk = (rng.integers(0, dom, nr) - dom // 2).astype(kdt)
+    sk = (rng.integers(0, dom, ns) - dom // 2).astype(kdt)
+    if nr * ns > 0 and nr * ns * 1.0 / max(dom, 1) > 5e6:  # keep |J| bounded
+        sk = sk[: max(1, int(5e6 * dom / nr))]
+        ns = len(sk)
+    rp = rng.integers(-2**31, 2**31, nr).astype(np.int32 if rb == 32 else np.int64)
+    sp = rng.integers(-2**31, 2**31, ns).astype(np.int32 if sb == 32 else np.int64)
+    if rb == 64:
+        rp = rp * 7919 + (1 << 40)
+    j = joiner(DT[kb], DT[rb], DT[sb])
+    want = oracle_res(rk, rp, sk, sp, materialize=True)
+    n = want["count"]
+    out_r = torch.empty(max(n, 1), dtype=DT[rb], device="cuda")
+    out_s = torch.empty(max(n, 1), dtype=DT[sb], device="cuda")
+    res = j.join(cuda(rk), cuda(rp), cuda(sk), cuda(sp), out_r, out_s)
+    check(res, want)
+    assert res.n_written == n
+    a, b = sorted_pairs(out_r[:n], out_s[:n])
+    assert np.array_equal(a, want["pairs"][0]) and np.array_equal(b, want["pairs"][1])
+
+
+@pytest.mark.parametrize("cfg,nr,ns", [("c1", 1 << 20, 1 << 20), ("c2", 1 << 22, 1 << 22),
+                                       ("c2", (1 << 22) + 12345, (1 << 22) + 12345),
+                                       ("c3", 1 << 18, 1 << 21), ("c3", 100_003, 700_001),
+                                       ("c5", 1 << 18, 1 << 20)])
+def test_config_recipes_vs_oracle(cfg, nr, ns):
+    wl = datagen.make(cfg, n_r=nr, n_s=ns)
+    kdt = DT[wl.key_bits]
+    want = oracle_res(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload)
+    j = joiner(kdt)
+    res = j.join(cuda(wl.R.key), cuda(wl.R.payload), cuda(wl.S.key), cuda(wl.S.payload))
+    check(res, want)
+    assert res.match_count == ns  # closed form (P793-794)
+
+
+def test_c1_full_with_pairs_vs_oracle():
+    wl = datagen.make("c1")
+    want = oracle_res(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload, materialize=True)
+    j = joiner(torch.int32)
+    n = want["count"]
+    out_r = torch.empty(n, dtype=torch.int32, device="cuda")
+    out_s = torch.empty(n, dtype=torch.int32, device="cuda")
+    res = j.join(cuda(wl.R.key), cuda(wl.R.payload), cuda(wl.S.key), cuda(wl.S.payload), out_r, out_s)
+    check(res, want)
+    a, b = sorted_pairs(out_r, out_s)
+    assert np.array_equal(a, want["pairs"][0]) and np.array_equal(b, want["pairs"][1])
+
+
+@pytest.mark.parametrize("passes,bits", [(1, (0, 0)), (1, (4, 0)), (1, (11, 0)), (2, (3, 5)),
+                                         (2, (8, 8)), (2, (12, 2)), (2, (6, 12))])
+def test_metamorphic_plans_identical(passes, bits):
+    wl = datagen.make("c2", n_r=1 << 20, n_s=(1 << 20) + 3)
+    ref = provenance.expected_from_workload(wl)
+    j = joiner(torch.int32, radix_passes=passes, radix_bits=bits)
+    res = j.join(cuda(wl.R.key), cuda(wl.R.payload), cuda(wl.S.key), cuda(wl.S.payload))
+    check(res, ref)
+    assert res.passes == passes
+
+
+def test_duplicate_heavy_and_oversized_partitions():
+    # R partitions far larger than the smem build capacity (R-chunking) and
+    # huge S partitions (S-slices): all keys in a handful of values
+    rng = np.random.default_rng(5)
+    rk = rng.integers(0, 3, 20000).astype(np.int32)
+    sk = rng.integers(0, 4, 50000).astype(np.int32)
+    rp = rng.integers(-100, 100, 20000).astype(np.int32)
+    sp = rng.integers(-100, 100, 50000).astype(np.int32)
+    want = oracle_res(rk, rp, sk, sp)
+    res = joiner(torch.int32).join(cuda(rk), cuda(rp), cuda(sk), cuda(sp))
+    check(res, want)
+    # all-equal keys: a*b
+    a, b = 5000, 3000
+    res = joiner(torch.int64).join(cuda(np.full(a, -7, np.int64)), cuda(np.arange(a)),
+                                   cuda(np.full(b, -7, np.int64)), cuda(np.arange(b)))
+    assert res.match_count == a * b
+    assert res.sum_r_payload == (b * (a * (a - 1) // 2)) & M64
+
+
+def test_extreme_keys():
+    for kdt in (np.int32, np.int64):
+        info = np.iinfo(kdt)
+        vals = np.array([info.min, info.max, -1, 0, 1, info.min + 1, info.max - 1], kdt)
+        rng = np.random.default_rng(3)
+        rk = rng.choice(vals, 3000).astype(kdt)
+        sk = rng.choice(vals, 5000).astype(kdt)
+        rp = np.arange(3000).astype(kdt)
+        sp = np.arange(5000).astype(kdt)
+        want = oracle_res(rk, rp, sk, sp)
+        res = joiner(torch.from_numpy(rk).dtype).join(cuda(rk), cuda(rp), cuda(sk), cuda(sp))
+        check(res, want)
+
+
+def test_empty_inputs():
+    e32 = torch.empty(0, dtype=torch.int32, device="cuda")
+    x = torch.arange(100, dtype=torch.int32, device="cuda")
+    j = joiner(torch.int32)
+    for args in ((e32, e32, x, x), (x, x, e32, e32), (e32, e32, e32, e32)):
+        res = j.join(*args)
+        assert res.as_tuple() == (0, 0, 0, 0)
+
+
+def test_output_capacity_protocol():
+    wl = datagen.make("c1", n_r=1 << 16, n_s=1 << 16)
+    want = provenance.expected_from_workload(wl)
+    j = joiner(torch.int32)
+    out_r = torch.empty(1000, dtype=torch.int32, device="cuda")
+    out_s = torch.empty(1000, dtype=torch.int32, device="cuda")
+    args = (cuda(wl.R.key), cuda(wl.R.payload), cuda(wl.S.key), cuda(wl.S.payload))
+    with pytest.raises(HapeError) as ei:
+        j.join(*args, out_r, out_s)
+    assert ei.value.status == _lib.HAPE_ERR_OUTPUT_CAPACITY
+    res = j.join(*args, out_r, out_s, raise_on_capacity=False)
+    check(res, want)
+    assert res.n_required == 1 << 16 and res.n_written == 1000
+    # the written prefix is a sub-multiset of J: every pair is a real match
+    rp = np.asarray(wl.R.payload)
+    pairs_ok = set(zip(rp[wl.idx.astype(np.int64)].tolist(), wl.S.payload.tolist()))
+    got = set(zip(out_r.cpu().tolist(), out_s.cpu().tolist()))
+    assert got <= pairs_ok and len(got) == 1000
+
+
+def test_host_resident_inputs_and_outputs():
+    wl = datagen.make("c3", n_r=1 << 15, n_s=1 << 17)
+    want = oracle_res(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload, materialize=True)
+    pin = lambda a: torch.from_numpy(np.ascontiguousarray(a)).pin_memory()
+    n = want["count"]
+    out_r = torch.empty(n, dtype=torch.int64).pin_memory()
+    out_s = torch.empty(n, dtype=torch.int64).pin_memory()
+    res = joiner(torch.int64).join(pin(wl.R.key), pin(wl.R.payload), pin(wl.S.key), pin(wl.S.payload),
+                                   out_r, out_s)
+    check(res, want)
+    a, b = sorted_pairs(out_r, out_s)
+    assert np.array_equal(a, want["pairs"][0]) and np.array_equal(b, want["pairs"][1])
+    assert res.stage_ms["h2d"] > 0
+
+
+def test_invalid_args():
+    j = joiner(torch.int32)
+    x = torch.arange(10, dtype=torch.int32, device="cuda")
+    R = _lib.hape_relation(None, None, 10, 0)
+    S = _lib.hape_relation(x.data_ptr(), x.data_ptr(), 10, 0)
+    res = _lib.hape_join_result()
+    assert _lib.hape_radix_join(j.handle, R, S, None, res) == _lib.HAPE_ERR_INVALID_ARG
+    R = _lib.hape_relation(x.data_ptr() + 1, x.data_ptr(), 9, 0)  # misaligned
+    assert _lib.hape_radix_join(j.handle, R, S, None, res) == _lib.HAPE_ERR_INVALID_ARG
+    R = _lib.hape_relation(x.data_ptr(), x.data_ptr(), 10, 7)     # bad mem kind
+    assert _lib.hape_radix_join(j.handle, R, S, None, res) == _lib.HAPE_ERR_INVALID_ARG
+    assert "mem" in _lib.hape_last_error(j.handle)
+
+
+# ---- stage invariants (a6-a9) through the debug entry point -----------------
+@pytest.mark.parametrize("passes,bits,kb", [(1, (9, 0), 32), (2, (8, 8), 32), (2, (5, 7), 64),
+                                            (1, (12, 0), 64)])
+def test_partition_invariants(passes, bits, kb):
+    n = (1 << 20) + 777
+    rng = np.random.default_rng(11)
+    kdt = np.int32 if kb == 32 else np.int64
+    keys = rng.integers(np.iinfo(kdt).min, np.iinfo(kdt).max, n, dtype=kdt)
+    pays = np.arange(n).astype(kdt)
+    j = joiner(DT[kb], radix_passes=passes, radix_bits=bits)
+    ok, op, ob, plan = j.debug_partition(cuda(keys), cuda(pays))
+    ok, op, ob = ok.cpu().numpy(), op.cpu().numpy(), ob.cpu().numpy()
+    b1, b2 = bits
+    Q = 1 << (b1 + (b2 if passes == 2 else 0))
+    # bounds monotone, start at 0, end at N; histogram sums to N
+    assert ob[0] == 0 and ob[-1] == n and np.all(np.diff(ob) >= 0) and len(ob) == Q + 1
+    # permutation: payload column is a permutation of 0..n-1 and pairs stay together
+    assert np.array_equal(np.sort(op), pays)
+    assert np.array_equal(ok, keys[op.astype(np.int64)])
+    # every tuple in partition q has partition_id(key) == q
+    pid = partition.partition_id(ok, b1, b2 if passes == 2 else 0)
+    expect = np.repeat(np.arange(Q), np.diff(ob))
+    assert np.array_equal(pid, expect)
+    # per-partition counts equal np.bincount of the partition function
+    assert np.array_equal(np.diff(ob), np.bincount(partition.partition_id(keys, b1, b2 if passes == 2 else 0),
+                                                   minlength=Q))
+
+
+def test_identity_partitions_equal_size():
+    # P802-804: "we select the keys so that all produced partitions have
+    # exactly the same size" -- dense keys + identity partition function
+    n = 1 << 21
+    keys = np.random.default_rng(2).permutation(n).astype(np.int32)
+    j = joiner(torch.int32, radix_passes=2, radix_bits=(6, 5), identity=True)
+    ok, op, ob, _ = j.debug_partition(cuda(keys), cuda(keys))
+    assert np.all(np.diff(ob.cpu().numpy()) == n >> 11)
+    wl = datagen.make("c1", n_r=n, n_s=n)
+    res = j.join(cuda(wl.R.key), cuda(wl.R.payload), cuda(wl.S.key), cuda(wl.S.payload))
+    check(res, provenance.expected_from_workload(wl))
