@@ -127,12 +127,12 @@ def fmix64(x: np.ndarray) -> np.ndarray:
 
 
 def mix(p: np.ndarray, q: np.ndarray) -> np.ndarray:
-    """mix(p, q) = fmix64((u64)p * 0x9E3779B97F4A7C15 + fmix64((u64)q)),
+    """mix(p, q) = fmix64((u64)p * 0x9E3779B97F4A7C15 + (u64)q),
     p and q sign-extended to 64 bits first (R10)."""
     pu = np.asarray(p).astype(np.int64).view(np.uint64)
     qu = np.asarray(q).astype(np.int64).view(np.uint64)
     with np.errstate(over="ignore"):
-        return fmix64(pu * _U(0x9E3779B97F4A7C15) + fmix64(qu))
+        return fmix64(pu * _U(0x9E3779B97F4A7C15) + qu)
 
 
 def u64sum(x: np.ndarray) -> int:

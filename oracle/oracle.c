@@ -19,7 +19,7 @@
  *   sum_r         = sum over J of (u64)(i64) p      (mod 2^64)
  *   sum_s         = sum over J of (u64)(i64) q      (mod 2^64)
  *   pair_checksum = sum over J of mix(p, q)         (mod 2^64)
- *   mix(p, q)     = fmix64((u64)p * 0x9E3779B97F4A7C15 + fmix64((u64)q))
+ *   mix(p, q)     = fmix64((u64)p * 0x9E3779B97F4A7C15 + (u64)q)
  *   fmix64        = the splitmix64 finaliser
  * Readings of the paper's silences (bag semantics, sign extension, wrapping
  * u64 sums, pair_checksum itself) are DESIGN.md readings R5/R6/R8/R10.
@@ -44,7 +44,7 @@ static uint64_t oracle_fmix64(uint64_t x) {
 }
 
 uint64_t oracle_mix(int64_t p, int64_t q) {
-  return oracle_fmix64((uint64_t)p * 0x9E3779B97F4A7C15ULL + oracle_fmix64((uint64_t)q));
+  return oracle_fmix64((uint64_t)p * 0x9E3779B97F4A7C15ULL + (uint64_t)q);
 }
 
 uint64_t oracle_fmix64_export(uint64_t x) { return oracle_fmix64(x); }

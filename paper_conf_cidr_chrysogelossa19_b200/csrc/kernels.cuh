@@ -62,9 +62,9 @@ __device__ __forceinline__ uint32_t bucket_of(uint64_t h, BitField bf) {
   return (uint32_t)(h >> bf.shift) & bf.mask;
 }
 
-// pair-checksum term (R10): mix(p,q) = fmix64(p*phi + fmix64(q))
+// pair-checksum term (R10): mix(p,q) = fmix64(p*phi + q)
 __device__ __forceinline__ uint64_t pair_mix(int64_t p, int64_t q) {
-  return fmix64((uint64_t)p * 0x9E3779B97F4A7C15ull + fmix64((uint64_t)q));
+  return fmix64((uint64_t)p * 0x9E3779B97F4A7C15ull + (uint64_t)q);
 }
 
 // --------------------------------------------------------------------------
@@ -137,6 +137,7 @@ __device__ uint32_t block_exscan_smem(uint32_t* a, int n, uint32_t* wtmp) {
 // the per-row totals rowsum[seg*P + p].
 // --------------------------------------------------------------------------
 constexpr int HIST_THREADS = 512;
+constexpr int HIST_VEC = 4;  // 16-byte loads in flight per thread per iteration
 
 template <int KW>
 __global__ void __launch_bounds__(HIST_THREADS)
@@ -144,20 +145,39 @@ k_hist(const typename UW<KW>::T* __restrict__ key, SegMap m, BitField bf, int id
        uint32_t* __restrict__ hist, uint32_t* __restrict__ rowsum) {
   extern __shared__ uint32_t sh_cnt[];
   using K = typename UW<KW>::T;
+  constexpr int PER = 16 / KW;  // keys per 16-byte vector
   for (uint32_t i = threadIdx.x; i < P; i += HIST_THREADS) sh_cnt[i] = 0;
   __syncthreads();
   uint32_t seg, j, lo, hi;
   seg_chunk(m, blockIdx.x, seg, j, lo, hi);
-  constexpr int U = 4;
-  uint32_t i = lo + threadIdx.x;
-  for (; i + (U - 1) * HIST_THREADS < hi; i += U * HIST_THREADS) {
-    K k[U];
+  // scalar head up to a 16-byte boundary, 16-byte vector body, scalar tail
+  uint32_t vlo = lo;
+  while (vlo < hi && (reinterpret_cast<uintptr_t>(key + vlo) & 15)) vlo++;
+  const uint32_t nvec = (hi - vlo) / PER;
+  const uint32_t vhi = vlo + nvec * PER;
+  for (uint32_t i = lo + threadIdx.x; i < vlo; i += HIST_THREADS)
+    atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(key[i], ident), bf)], 1u);
+  for (uint32_t i = vhi + threadIdx.x; i < hi; i += HIST_THREADS)
+    atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(key[i], ident), bf)], 1u);
+  const uint4* __restrict__ vk = reinterpret_cast<const uint4*>(key + vlo);
+  uint32_t v = threadIdx.x;
+  for (; v + (HIST_VEC - 1) * HIST_THREADS < nvec; v += HIST_VEC * HIST_THREADS) {
+    uint4 w[HIST_VEC];
 #pragma unroll
-    for (int u = 0; u < U; u++) k[u] = __ldcs(key + i + u * HIST_THREADS);
+    for (int u = 0; u < HIST_VEC; u++) w[u] = __ldcs(vk + v + u * HIST_THREADS);
 #pragma unroll
-    for (int u = 0; u < U; u++) atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(k[u], ident), bf)], 1u);
+    for (int u = 0; u < HIST_VEC; u++) {
+      const K* kk = reinterpret_cast<const K*>(&w[u]);
+#pragma unroll
+      for (int e = 0; e < PER; e++) atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(kk[e], ident), bf)], 1u);
+    }
   }
-  for (; i < hi; i += HIST_THREADS) atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(__ldcs(key + i), ident), bf)], 1u);
+  for (; v < nvec; v += HIST_THREADS) {
+    const uint4 w = __ldcs(vk + v);
+    const K* kk = reinterpret_cast<const K*>(&w);
+#pragma unroll
+    for (int e = 0; e < PER; e++) atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(kk[e], ident), bf)], 1u);
+  }
   __syncthreads();
   const uint32_t row0 = seg * P;
   for (uint32_t p = threadIdx.x; p < P; p += HIST_THREADS) {
@@ -224,13 +244,62 @@ k_scan(uint32_t* __restrict__ hist, const uint32_t* __restrict__ rowsum, SegMap 
 // of one bucket continue where the previous tile's stopped, so L2 merges
 // partial sectors before they reach HBM).
 // --------------------------------------------------------------------------
+// The raw input tiles are streamed into shared memory by the bulk-copy
+// engine (cp.async.bulk, TMA 1-D) into a ring of SC_STAGES buffers tracked by
+// mbarriers, so HBM reads overlap the ranking / reordering / write-out of the
+// previous tile.  Tiles start at arbitrary element offsets: the copy covers
+// the enclosing 16-byte-aligned byte range and the tile is read at an offset.
 constexpr int SC_THREADS = 512;
-constexpr int SC_ITEMS = 8;
-constexpr int SC_TILE = SC_THREADS * SC_ITEMS;
+constexpr int SC_STAGES = 2;
+
+template <int KW, int PW> struct ScTile { static constexpr int T = (KW + PW) <= 8 ? 4096 : 2048; };
+
+__device__ __forceinline__ uint32_t smem_u32(const void* p) {
+  return static_cast<uint32_t>(__cvta_generic_to_shared(p));
+}
+__device__ __forceinline__ void mbar_init(uint64_t* bar, uint32_t count) {
+  asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count));
+}
+__device__ __forceinline__ void mbar_expect_tx(uint64_t* bar, uint32_t bytes) {
+  asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes)
+               : "memory");
+}
+__device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t phase) {
+  asm volatile(
+      "{\n .reg .pred p;\n WAIT_%=:\n"
+      " mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n"
+      " @!p bra WAIT_%=;\n}\n" ::"r"(smem_u32(bar)),
+      "r"(phase)
+      : "memory");
+}
+__device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes, uint64_t* bar) {
+  asm volatile(
+      "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
+          smem_u32(dst)),
+      "l"(src), "r"(bytes), "r"(smem_u32(bar))
+      : "memory");
+}
 
 template <int KW, int PW>
 __host__ __device__ constexpr size_t scatter_smem_bytes(uint32_t P) {
-  return (size_t)SC_TILE * (KW + PW + 2) + (size_t)P * 12 + 33 * 4;
+  constexpr int T = ScTile<KW, PW>::T;
+  return (size_t)SC_STAGES * ((size_t)T * KW + 32 + (size_t)T * PW + 32)  // raw ring
+         + (size_t)T * (KW + PW + 2)                                        // reordered tile
+         + (size_t)P * 16 + 64 * 4 + SC_STAGES * 8 + 64;
+}
+
+// issue the bulk copies of tile [t0, t0+tn) into ring stage s; returns nothing,
+// the consumer recomputes the in-buffer element offsets
+template <int KW, int PW>
+__device__ __forceinline__ void sc_issue(const void* ik, const void* ip, uint32_t t0, uint32_t tn,
+                                         unsigned char* rk, unsigned char* rp, uint64_t* bar) {
+  const uintptr_t ka = reinterpret_cast<uintptr_t>(ik) + (uintptr_t)t0 * KW;
+  const uintptr_t pa = reinterpret_cast<uintptr_t>(ip) + (uintptr_t)t0 * PW;
+  const uintptr_t k0 = ka & ~(uintptr_t)15, k1 = (ka + (uintptr_t)tn * KW + 15) & ~(uintptr_t)15;
+  const uintptr_t p0 = pa & ~(uintptr_t)15, p1 = (pa + (uintptr_t)tn * PW + 15) & ~(uintptr_t)15;
+  mbar_expect_tx(bar, (uint32_t)((k1 - k0) + (p1 - p0)));
+  bulk_g2s(rk, reinterpret_cast<const void*>(k0), (uint32_t)(k1 - k0), bar);
+  bulk_g2s(rp, reinterpret_cast<const void*>(p0), (uint32_t)(p1 - p0), bar);
 }
 
 template <int KW, int PW>
@@ -240,72 +309,108 @@ k_scatter(const typename UW<KW>::T* __restrict__ ik, const typename UW<PW>::T* _
           typename UW<KW>::T* __restrict__ ok, typename UW<PW>::T* __restrict__ op) {
   using K = typename UW<KW>::T;
   using V = typename UW<PW>::T;
-  extern __shared__ __align__(16) unsigned char smem[];
-  K* s_key = reinterpret_cast<K*>(smem);
-  V* s_pay = reinterpret_cast<V*>(smem + (size_t)SC_TILE * KW);
-  uint16_t* s_bkt = reinterpret_cast<uint16_t*>(smem + (size_t)SC_TILE * (KW + PW));
-  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(smem + (size_t)SC_TILE * (KW + PW + 2));
-  uint32_t* s_cur = s_cnt + P;     // running absolute write cursor per bucket
-  uint32_t* s_dlt = s_cur + P;     // cursor - tile start of the bucket
-  uint32_t* wtmp = s_dlt + P;
+  constexpr int T = ScTile<KW, PW>::T;
+  constexpr int ITEMS = T / SC_THREADS;
+  constexpr int RK = T * KW + 32, RP = T * PW + 32;
+  extern __shared__ __align__(128) unsigned char smem[];
+  unsigned char* raw = smem;                                            // [S][RK | RP]
+  K* s_key = reinterpret_cast<K*>(smem + SC_STAGES * (RK + RP));
+  V* s_pay = reinterpret_cast<V*>(reinterpret_cast<unsigned char*>(s_key) + (size_t)T * KW);
+  uint16_t* s_bkt = reinterpret_cast<uint16_t*>(reinterpret_cast<unsigned char*>(s_pay) + (size_t)T * PW);
+  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_bkt + T);
+  uint32_t* s_st = s_cnt + P;    // tile start of the bucket's run
+  uint32_t* s_cur = s_st + P;    // absolute write cursor
+  uint32_t* s_dlt = s_cur + P;   // cursor - tile start
+  uint32_t* s_wt = s_dlt + P;    // warp totals [16]
+  uint64_t* bar = reinterpret_cast<uint64_t*>(s_wt + 64);
 
   uint32_t seg, j, lo, hi;
   seg_chunk(m, blockIdx.x, seg, j, lo, hi);
   const uint32_t row0 = seg * P;
-  for (uint32_t p = threadIdx.x; p < P; p += SC_THREADS)
+  const uint32_t ntiles = (hi - lo + T - 1) / T;
+  for (uint32_t p = threadIdx.x; p < P; p += SC_THREADS) {
     s_cur[p] = offsets[(size_t)(row0 + p) * m.cps + j];
+    s_cnt[p] = 0;
+  }
+  if (threadIdx.x == 0) {
+    for (int s = 0; s < SC_STAGES; s++) mbar_init(&bar[s], 1);
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    for (uint32_t t = 0; t < (uint32_t)SC_STAGES && t < ntiles; t++) {
+      const uint32_t t0 = lo + t * T;
+      sc_issue<KW, PW>(ik, ip, t0, min((uint32_t)T, hi - t0), raw + t * (RK + RP), raw + t * (RK + RP) + RK, &bar[t]);
+    }
+  }
+  __syncthreads();
 
-  for (uint32_t t0 = lo; t0 < hi; t0 += SC_TILE) {
-    const uint32_t tn = min((uint32_t)SC_TILE, hi - t0);
-    for (uint32_t p = threadIdx.x; p < P; p += SC_THREADS) s_cnt[p] = 0;
-    __syncthreads();
-    K k[SC_ITEMS];
-    V v[SC_ITEMS];
-    uint32_t b[SC_ITEMS], r[SC_ITEMS];
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  constexpr int NW = SC_THREADS / 32;
+  for (uint32_t t = 0; t < ntiles; t++) {
+    const uint32_t s = t % SC_STAGES, ph = (t / SC_STAGES) & 1;
+    const uint32_t t0 = lo + t * T, tn = min((uint32_t)T, hi - t0);
+    const unsigned char* rk = raw + s * (RK + RP);
+    const unsigned char* rp = rk + RK;
+    const K* tk = reinterpret_cast<const K*>(rk + ((reinterpret_cast<uintptr_t>(ik) + (uintptr_t)t0 * KW) & 15));
+    const V* tp = reinterpret_cast<const V*>(rp + ((reinterpret_cast<uintptr_t>(ip) + (uintptr_t)t0 * PW) & 15));
+    mbar_wait(&bar[s], ph);
+    // phase 1: bucket + rank (shared-memory atomic claim)
+    uint32_t br[ITEMS];
 #pragma unroll
-    for (int u = 0; u < SC_ITEMS; u++) {
-      const uint32_t i = u * SC_THREADS + threadIdx.x;
-      if (i < tn) { k[u] = __ldcs(ik + t0 + i); v[u] = __ldcs(ip + t0 + i); }
-    }
-#pragma unroll
-    for (int u = 0; u < SC_ITEMS; u++) {
-      const uint32_t i = u * SC_THREADS + threadIdx.x;
-      if (i < tn) {
-        b[u] = bucket_of(part_hash<KW>(k[u], ident), bf);
-        r[u] = atomicAdd(&s_cnt[b[u]], 1u);
-      }
-    }
-    __syncthreads();
-    // tile start of every bucket; delta = where the bucket's run goes in HBM
-    // minus where it sits in the reordered tile
-    for (uint32_t p = threadIdx.x; p < P; p += SC_THREADS) s_dlt[p] = s_cnt[p];
-    __syncthreads();
-    block_exscan_smem<SC_THREADS>(s_dlt, (int)P, wtmp);  // s_dlt = tile start
-    for (uint32_t p = threadIdx.x; p < P; p += SC_THREADS) {
-      const uint32_t st = s_dlt[p], c = s_cnt[p], cur = s_cur[p];
-      s_dlt[p] = cur - st;
-      s_cnt[p] = st;                                     // keep the start for placement
-      s_cur[p] = cur + c;
-    }
-    __syncthreads();
-#pragma unroll
-    for (int u = 0; u < SC_ITEMS; u++) {
+    for (int u = 0; u < ITEMS; u++) {
       const uint32_t i = u * SC_THREADS + threadIdx.x;
       if (i < tn) {
-        const uint32_t pos = s_cnt[b[u]] + r[u];
-        s_key[pos] = k[u];
-        s_pay[pos] = v[u];
-        s_bkt[pos] = (uint16_t)b[u];
+        const uint32_t b = bucket_of(part_hash<KW>(tk[i], ident), bf);
+        br[u] = (b << 16) | atomicAdd(&s_cnt[b], 1u);
       }
     }
-    __syncthreads();
+    __syncthreads();  // A
+    // phase 2: exclusive scan of the tile's bucket counts (one bucket run per
+    // thread group), advance the per-bucket HBM cursors
+    {
+      const uint32_t per = (P + SC_THREADS - 1) / SC_THREADS;
+      const uint32_t b0 = min(threadIdx.x * per, P), b1 = min(b0 + per, P);
+      uint32_t sum = 0;
+      for (uint32_t b = b0; b < b1; b++) sum += s_cnt[b];
+      const uint32_t inc = warp_incl_scan(sum);
+      if (lane == 31) s_wt[warp] = inc;
+      __syncthreads();  // X
+      uint32_t ex = inc - sum;
+      for (int w = 0; w < warp; w++) ex += s_wt[w];
+      for (uint32_t b = b0; b < b1; b++) {
+        const uint32_t c = s_cnt[b], cur = s_cur[b];
+        s_st[b] = ex;
+        s_dlt[b] = cur - ex;
+        s_cur[b] = cur + c;
+        s_cnt[b] = 0;
+        ex += c;
+      }
+    }
+    __syncthreads();  // B
+    // phase 3: reorder the tile in shared memory, bucket runs consecutive
+#pragma unroll
+    for (int u = 0; u < ITEMS; u++) {
+      const uint32_t i = u * SC_THREADS + threadIdx.x;
+      if (i < tn) {
+        const uint32_t b = br[u] >> 16;
+        const uint32_t pos = s_st[b] + (br[u] & 0xFFFFu);
+        s_key[pos] = tk[i];
+        s_pay[pos] = tp[i];
+        s_bkt[pos] = (uint16_t)b;
+      }
+    }
+    __syncthreads();  // C: raw stage s is free, the reordered tile is complete
+    if (threadIdx.x == 0 && t + SC_STAGES < ntiles) {
+      const uint32_t n0 = lo + (t + SC_STAGES) * T;
+      sc_issue<KW, PW>(ik, ip, n0, min((uint32_t)T, hi - n0), raw + s * (RK + RP), raw + s * (RK + RP) + RK, &bar[s]);
+    }
+    // phase 4: write the runs; consecutive threads -> consecutive addresses
+#pragma unroll 4
     for (uint32_t i = threadIdx.x; i < tn; i += SC_THREADS) {
       const uint32_t dst = s_dlt[s_bkt[i]] + i;
-      ok[dst] = s_key[i];
-      op[dst] = s_pay[i];
+      __stcs(ok + dst, s_key[i]);
+      __stcs(op + dst, s_pay[i]);
     }
-    __syncthreads();
   }
+  (void)NW;
 }
 
 // --------------------------------------------------------------------------
@@ -449,14 +554,23 @@ k_build_probe(JoinArgs a) {
         uint32_t c[JN_U];
 #pragma unroll
         for (int u = 0; u < JN_U; u++) {
+          // walk the chain to the next match (cheap, divergent), then run the
+          // aggregation body once per round for all lanes that found one
+          // (converged), so the checksum's 64-bit mixing is not replayed per
+          // divergent chain position
           c[u] = 0;
-          for (uint32_t e = head[u]; e != JN_NIL; e = s_next[e]) {
-            if (s_rk[e] == k[u]) {
+          uint32_t e = head[u];
+          while (true) {
+            while (e != JN_NIL && s_rk[e] != k[u]) e = s_next[e];
+            const bool hit = e != JN_NIL;
+            if (!__any_sync(0xffffffffu, hit)) break;
+            if (hit) {
               const int64_t pr = (int64_t)s_rp[e], ps = (int64_t)v[u];
               c[u]++;
               sr += (unsigned long long)pr;
               ss += (unsigned long long)ps;
               sx += pair_mix(pr, ps);
+              e = s_next[e];
             }
           }
           cnt += c[u];

@@ -29,7 +29,7 @@ def _py_fmix64(x):
 
 
 def _py_mix(p, q):
-    return _py_fmix64((p & M64) * 0x9E3779B97F4A7C15 + _py_fmix64(q & M64))
+    return _py_fmix64((p & M64) * 0x9E3779B97F4A7C15 + (q & M64))
 
 
 def brute(rk, rp, sk, sp):
