@@ -17,6 +17,7 @@
 #include <algorithm>
 #include <cstdarg>
 #include <cstdio>
+#include <cstdlib>
 #include <cstring>
 #include <string>
 #include <vector>
@@ -185,15 +186,29 @@ static hape_status make_plan(const hape_join* h, uint64_t n_r, uint64_t n_s, hap
   p->bits[1] = b2;
   const uint64_t Q = 1ull << (b1 + b2);
   const uint64_t expected = (n_r + Q - 1) / Q;
-  uint64_t cap = expected + expected / 4 + 128;
-  cap = std::max<uint64_t>(512, std::min<uint64_t>(cap, 8192));
-  cap = (cap + 255) & ~255ull;
+  // R chunk capacity: mean + 12.5% (+64) covers the hash spread of a uniform
+  // co-partition (sigma = sqrt(mean)); larger co-partitions are chunked (R6)
+  // R chunk capacity: mean + 12.5% (+64) covers the hash spread of a uniform
+  // co-partition (sigma = sqrt(mean)); larger co-partitions are chunked (R6).
+  // Heads: 2^sb >= ~2x the chunk (load factor ~0.5); HAPE_SLOT_EXTRA (tuning)
+  // shifts the exponent.  Both shrink until the table fits ~2 CTAs per SM.
+  int extra = 0;
+  if (const char* e = getenv("HAPE_SLOT_EXTRA")) extra = atoi(e);
+  const int prw = pay_width(c.r_payload_type), kwb = key_width(c);
+  uint64_t cap = expected + expected / 8 + 64;
+  cap = std::max<uint64_t>(256, std::min<uint64_t>(cap, JN_MAXCAP));
+  cap = (cap + 127) & ~127ull;
+  uint32_t sb = 0;
+  while (true) {
+    const int sbi = (int)ceil_log2_u64(std::min<uint64_t>(std::max<uint64_t>(expected, 1), cap)) + extra;
+    sb = (uint32_t)std::max(6, std::min(sbi, 14));
+    const size_t bytes = 2 * ((cap * kwb + 47) / 16 * 16 + (cap * prw + 47) / 16 * 16) + (cap * 2 + 15) / 16 * 16 +
+                         ((size_t)4 << sb);
+    if (bytes <= 110 * 1024 || cap <= 256) break;
+    cap -= 128;
+  }
   p->build_cap = (uint32_t)cap;
-  uint32_t sb = ceil_log2_u64(cap);
-  sb = std::max(6u, std::min(sb, 14u));
-  p->slot_shift = b1 + b2;
-  const int avail = (int)HW - (int)p->dest_bits - (int)p->slot_shift;
-  if ((int)sb > avail) sb = (uint32_t)std::max(0, avail);
+  p->slot_shift = 0;  // slots use a multiplicative hash of the key (kernels.cuh jn_slot)
   p->slot_bits = sb;
   p->probe_slice = 16384;
   p->ctas_per_seg[0] = cps_for(h, n_r, 1);

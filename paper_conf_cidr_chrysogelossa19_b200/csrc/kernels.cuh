@@ -129,6 +129,42 @@ __device__ uint32_t block_exscan_smem(uint32_t* a, int n, uint32_t* wtmp) {
   return total;
 }
 
+// Conflict-free exclusive scan of a[0..n) in shared memory by the first NT
+// threads: warp w owns a contiguous chunk and reads it lane-strided (one
+// word per bank per access); PACK writes (start | end << 16) instead of the
+// start.  wt: >= NT/32 words.  Two barriers (bar id 1 when NAMED, else 0).
+template <int NT, bool PACK, bool NAMED>
+__device__ __forceinline__ uint32_t block_exscan_strided(uint32_t* a, uint32_t n, uint32_t* wt) {
+  constexpr int NW = NT / 32;
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  const uint32_t chunk = ((n + NW - 1) / NW + 31) & ~31u;
+  const uint32_t c0 = min(n, warp * chunk), c1 = min(n, c0 + chunk);
+  uint32_t s = 0;
+  for (uint32_t i = c0 + lane; i < c1; i += 32) s += a[i];
+#pragma unroll
+  for (int o = 16; o > 0; o >>= 1) s += __shfl_xor_sync(0xffffffffu, s, o);
+  if (lane == 0) wt[warp] = s;
+  if constexpr (NAMED) asm volatile("bar.sync 1, %0;" ::"n"(NT) : "memory");
+  else __syncthreads();
+  uint32_t carry = 0, total = 0;
+  for (int w = 0; w < NW; w++) {
+    const uint32_t x = wt[w];
+    carry += w < warp ? x : 0u;
+    total += x;
+  }
+  for (uint32_t b = c0; b < c1; b += 32) {
+    const uint32_t i = b + lane;
+    const uint32_t v = i < c1 ? a[i] : 0u;
+    const uint32_t inc = warp_incl_scan(v);
+    const uint32_t ex = carry + inc - v;
+    if (i < c1) a[i] = PACK ? (ex | ((ex + v) << 16)) : ex;
+    carry += __shfl_sync(0xffffffffu, inc, 31);
+  }
+  if constexpr (NAMED) asm volatile("bar.sync 1, %0;" ::"n"(NT) : "memory");
+  else __syncthreads();
+  return total;
+}
+
 // --------------------------------------------------------------------------
 // a6: radix histogram of one pass.  One contiguous chunk per CTA; keys only
 // (w_k bytes per tuple); shared-memory counters (P166-168: "use shared memory
@@ -221,7 +257,7 @@ k_scan(uint32_t* __restrict__ hist, const uint32_t* __restrict__ rowsum, SegMap 
     const int cn = (int)min((size_t)SCAN_TILE, e1 - c0);
     for (int i = threadIdx.x; i < cn; i += SCAN_THREADS) tile[i] = hist[c0 + i];
     __syncthreads();
-    uint32_t tot = block_exscan_smem<SCAN_THREADS>(tile, cn, wtmp);
+    uint32_t tot = block_exscan_strided<SCAN_THREADS, false, false>(tile, (uint32_t)cn, wtmp);
     for (int i = threadIdx.x; i < cn; i += SCAN_THREADS) {
       uint32_t off = carry + tile[i];
       hist[c0 + i] = off;
@@ -272,6 +308,20 @@ __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t phase) {
       "r"(phase)
       : "memory");
 }
+// producer-side wait: back off between polls so a warp that is far ahead
+// does not steal issue slots from the consumers
+__device__ __forceinline__ void mbar_wait_backoff(uint64_t* bar, uint32_t phase) {
+  uint32_t ok = 0;
+  while (true) {
+    asm volatile(
+        "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n selp.u32 %0, 1, 0, p;\n}\n"
+        : "=r"(ok)
+        : "r"(smem_u32(bar)), "r"(phase)
+        : "memory");
+    if (ok) return;
+    __nanosleep(256);
+  }
+}
 __device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes, uint64_t* bar) {
   asm volatile(
       "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
@@ -280,28 +330,54 @@ __device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t by
       : "memory");
 }
 
+__device__ __forceinline__ uint64_t policy_evict_first() {
+  uint64_t pol;
+  asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(pol));
+  return pol;
+}
+__device__ __forceinline__ void bulk_g2s_ef(void* dst, const void* src, uint32_t bytes, uint64_t* bar,
+                                            uint64_t pol) {
+  asm volatile(
+      "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.L2::cache_hint [%0], [%1], %2, [%3], %4;" ::"r"(
+          smem_u32(dst)),
+      "l"(src), "r"(bytes), "r"(smem_u32(bar)), "l"(pol)
+      : "memory");
+}
+
+// one reordered tuple in shared memory (a single random-position store)
+template <int KW, int PW>
+struct alignas((KW + PW) <= 8 ? 8 : 16) ScPair {
+  typename UW<KW>::T k;
+  typename UW<PW>::T v;
+};
+
 template <int KW, int PW>
 __host__ __device__ constexpr size_t scatter_smem_bytes(uint32_t P) {
   constexpr int T = ScTile<KW, PW>::T;
   return (size_t)SC_STAGES * ((size_t)T * KW + 32 + (size_t)T * PW + 32)  // raw ring
-         + (size_t)T * (KW + PW + 2)                                        // reordered tile
+         + (size_t)T * sizeof(ScPair<KW, PW>)                              // reordered tile
          + (size_t)P * 16 + 64 * 4 + SC_STAGES * 8 + 64;
 }
 
-// issue the bulk copies of tile [t0, t0+tn) into ring stage s; returns nothing,
-// the consumer recomputes the in-buffer element offsets
+// issue the bulk copies of tile [t0, t0+tn) into ring stage s (the enclosing
+// 16-byte-aligned byte ranges; the consumer reads at the residual offset)
 template <int KW, int PW>
 __device__ __forceinline__ void sc_issue(const void* ik, const void* ip, uint32_t t0, uint32_t tn,
-                                         unsigned char* rk, unsigned char* rp, uint64_t* bar) {
+                                         unsigned char* rk, unsigned char* rp, uint64_t* bar, uint64_t pol) {
   const uintptr_t ka = reinterpret_cast<uintptr_t>(ik) + (uintptr_t)t0 * KW;
   const uintptr_t pa = reinterpret_cast<uintptr_t>(ip) + (uintptr_t)t0 * PW;
   const uintptr_t k0 = ka & ~(uintptr_t)15, k1 = (ka + (uintptr_t)tn * KW + 15) & ~(uintptr_t)15;
   const uintptr_t p0 = pa & ~(uintptr_t)15, p1 = (pa + (uintptr_t)tn * PW + 15) & ~(uintptr_t)15;
   mbar_expect_tx(bar, (uint32_t)((k1 - k0) + (p1 - p0)));
-  bulk_g2s(rk, reinterpret_cast<const void*>(k0), (uint32_t)(k1 - k0), bar);
-  bulk_g2s(rp, reinterpret_cast<const void*>(p0), (uint32_t)(p1 - p0), bar);
+  bulk_g2s_ef(rk, reinterpret_cast<const void*>(k0), (uint32_t)(k1 - k0), bar, pol);
+  bulk_g2s_ef(rp, reinterpret_cast<const void*>(p0), (uint32_t)(p1 - p0), bar, pol);
 }
 
+// Odd chunks fill their per-bucket regions back to front: the sector shared
+// by the end of region (p, j) and the start of region (p, j+1) is then written
+// by both neighbours at the same moment of their lifetimes (both at the start,
+// or both at the end), so L2 merges it instead of evicting a half-written
+// sector and paying a DRAM read-modify-write.
 template <int KW, int PW>
 __global__ void __launch_bounds__(SC_THREADS, 2)
 k_scatter(const typename UW<KW>::T* __restrict__ ik, const typename UW<PW>::T* __restrict__ ip,
@@ -309,41 +385,45 @@ k_scatter(const typename UW<KW>::T* __restrict__ ik, const typename UW<PW>::T* _
           typename UW<KW>::T* __restrict__ ok, typename UW<PW>::T* __restrict__ op) {
   using K = typename UW<KW>::T;
   using V = typename UW<PW>::T;
+  using Pair = ScPair<KW, PW>;
   constexpr int T = ScTile<KW, PW>::T;
   constexpr int ITEMS = T / SC_THREADS;
   constexpr int RK = T * KW + 32, RP = T * PW + 32;
   extern __shared__ __align__(128) unsigned char smem[];
   unsigned char* raw = smem;                                            // [S][RK | RP]
-  K* s_key = reinterpret_cast<K*>(smem + SC_STAGES * (RK + RP));
-  V* s_pay = reinterpret_cast<V*>(reinterpret_cast<unsigned char*>(s_key) + (size_t)T * KW);
-  uint16_t* s_bkt = reinterpret_cast<uint16_t*>(reinterpret_cast<unsigned char*>(s_pay) + (size_t)T * PW);
-  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_bkt + T);
+  Pair* s_pair = reinterpret_cast<Pair*>(smem + SC_STAGES * (RK + RP));
+  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_pair + T);
   uint32_t* s_st = s_cnt + P;    // tile start of the bucket's run
-  uint32_t* s_cur = s_st + P;    // absolute write cursor
-  uint32_t* s_dlt = s_cur + P;   // cursor - tile start
+  uint32_t* s_cur = s_st + P;    // absolute write cursor (next free / one past next free if backward)
+  uint32_t* s_dlt = s_cur + P;   // HBM run start - tile run start
   uint32_t* s_wt = s_dlt + P;    // warp totals [16]
   uint64_t* bar = reinterpret_cast<uint64_t*>(s_wt + 64);
 
   uint32_t seg, j, lo, hi;
   seg_chunk(m, blockIdx.x, seg, j, lo, hi);
+  const bool backward = (j & 1u) != 0;
   const uint32_t row0 = seg * P;
+  const size_t nflat = (size_t)m.nseg * P * m.cps;
   const uint32_t ntiles = (hi - lo + T - 1) / T;
   for (uint32_t p = threadIdx.x; p < P; p += SC_THREADS) {
-    s_cur[p] = offsets[(size_t)(row0 + p) * m.cps + j];
+    const size_t f = (size_t)(row0 + p) * m.cps + j;
+    s_cur[p] = backward ? (f + 1 < nflat ? offsets[f + 1] : m.n) : offsets[f];
     s_cnt[p] = 0;
   }
+  uint64_t pol = 0;
   if (threadIdx.x == 0) {
+    pol = policy_evict_first();
     for (int s = 0; s < SC_STAGES; s++) mbar_init(&bar[s], 1);
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
     for (uint32_t t = 0; t < (uint32_t)SC_STAGES && t < ntiles; t++) {
       const uint32_t t0 = lo + t * T;
-      sc_issue<KW, PW>(ik, ip, t0, min((uint32_t)T, hi - t0), raw + t * (RK + RP), raw + t * (RK + RP) + RK, &bar[t]);
+      sc_issue<KW, PW>(ik, ip, t0, min((uint32_t)T, hi - t0), raw + t * (RK + RP), raw + t * (RK + RP) + RK,
+                       &bar[t], pol);
     }
   }
   __syncthreads();
 
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-  constexpr int NW = SC_THREADS / 32;
   for (uint32_t t = 0; t < ntiles; t++) {
     const uint32_t s = t % SC_STAGES, ph = (t / SC_STAGES) & 1;
     const uint32_t t0 = lo + t * T, tn = min((uint32_t)T, hi - t0);
@@ -352,19 +432,20 @@ k_scatter(const typename UW<KW>::T* __restrict__ ik, const typename UW<PW>::T* _
     const K* tk = reinterpret_cast<const K*>(rk + ((reinterpret_cast<uintptr_t>(ik) + (uintptr_t)t0 * KW) & 15));
     const V* tp = reinterpret_cast<const V*>(rp + ((reinterpret_cast<uintptr_t>(ip) + (uintptr_t)t0 * PW) & 15));
     mbar_wait(&bar[s], ph);
-    // phase 1: bucket + rank (shared-memory atomic claim)
+    // phase 1: bucket + rank (shared-memory atomic claim); keys stay in registers
     uint32_t br[ITEMS];
+    K kr[ITEMS];
 #pragma unroll
     for (int u = 0; u < ITEMS; u++) {
       const uint32_t i = u * SC_THREADS + threadIdx.x;
       if (i < tn) {
-        const uint32_t b = bucket_of(part_hash<KW>(tk[i], ident), bf);
+        kr[u] = tk[i];
+        const uint32_t b = bucket_of(part_hash<KW>(kr[u], ident), bf);
         br[u] = (b << 16) | atomicAdd(&s_cnt[b], 1u);
       }
     }
     __syncthreads();  // A
-    // phase 2: exclusive scan of the tile's bucket counts (one bucket run per
-    // thread group), advance the per-bucket HBM cursors
+    // phase 2: exclusive scan of the tile's bucket counts; advance the cursors
     {
       const uint32_t per = (P + SC_THREADS - 1) / SC_THREADS;
       const uint32_t b0 = min(threadIdx.x * per, P), b1 = min(b0 + per, P);
@@ -377,9 +458,10 @@ k_scatter(const typename UW<KW>::T* __restrict__ ik, const typename UW<PW>::T* _
       for (int w = 0; w < warp; w++) ex += s_wt[w];
       for (uint32_t b = b0; b < b1; b++) {
         const uint32_t c = s_cnt[b], cur = s_cur[b];
+        const uint32_t run = backward ? cur - c : cur;
         s_st[b] = ex;
-        s_dlt[b] = cur - ex;
-        s_cur[b] = cur + c;
+        s_dlt[b] = run - ex;
+        s_cur[b] = backward ? cur - c : cur + c;
         s_cnt[b] = 0;
         ex += c;
       }
@@ -390,27 +472,30 @@ k_scatter(const typename UW<KW>::T* __restrict__ ik, const typename UW<PW>::T* _
     for (int u = 0; u < ITEMS; u++) {
       const uint32_t i = u * SC_THREADS + threadIdx.x;
       if (i < tn) {
-        const uint32_t b = br[u] >> 16;
-        const uint32_t pos = s_st[b] + (br[u] & 0xFFFFu);
-        s_key[pos] = tk[i];
-        s_pay[pos] = tp[i];
-        s_bkt[pos] = (uint16_t)b;
+        const uint32_t pos = s_st[br[u] >> 16] + (br[u] & 0xFFFFu);
+        Pair pr;
+        pr.k = kr[u];
+        pr.v = tp[i];
+        s_pair[pos] = pr;
       }
     }
     __syncthreads();  // C: raw stage s is free, the reordered tile is complete
     if (threadIdx.x == 0 && t + SC_STAGES < ntiles) {
       const uint32_t n0 = lo + (t + SC_STAGES) * T;
-      sc_issue<KW, PW>(ik, ip, n0, min((uint32_t)T, hi - n0), raw + s * (RK + RP), raw + s * (RK + RP) + RK, &bar[s]);
+      sc_issue<KW, PW>(ik, ip, n0, min((uint32_t)T, hi - n0), raw + s * (RK + RP), raw + s * (RK + RP) + RK,
+                       &bar[s], pol);
     }
     // phase 4: write the runs; consecutive threads -> consecutive addresses
+    // (the bucket is recomputed from the key: ALU is cheaper than another
+    // random shared-memory store + load)
 #pragma unroll 4
     for (uint32_t i = threadIdx.x; i < tn; i += SC_THREADS) {
-      const uint32_t dst = s_dlt[s_bkt[i]] + i;
-      __stcs(ok + dst, s_key[i]);
-      __stcs(op + dst, s_pay[i]);
+      const Pair pr = s_pair[i];
+      const uint32_t dst = s_dlt[bucket_of(part_hash<KW>(pr.k, ident), bf)] + i;
+      ok[dst] = pr.k;
+      op[dst] = pr.v;
     }
   }
-  (void)NW;
 }
 
 // --------------------------------------------------------------------------
@@ -455,13 +540,35 @@ k_worklist(const uint32_t* __restrict__ bR, const uint32_t* __restrict__ bS, uin
 // between builds.  The slot uses hash bits above the radix bits (every tuple
 // of a co-partition shares those).
 // --------------------------------------------------------------------------
-constexpr int JN_THREADS = 256;
+// Warp-specialised pipeline (the Blackwell producer/consumer idiom):
+//   * a producer warp walks this CTA's static share of the work list
+//     (items blockIdx.x, +gridDim.x, ...; co-partitions are near-uniform, so a
+//     static split balances), reads the item's bounds and streams each R chunk
+//     into a 2-deep ring of shared-memory buffers with the bulk-copy engine
+//     (cp.async.bulk + mbarrier), one "stage" per (R chunk, S slice);
+//   * 8 consumer warps build a chained table over the landed chunk (heads
+//     reset per stage, atomicExch on the heads, u16 next links) and probe the S
+//     slice, streaming S from HBM with 4 independent loads per thread.
+// The next stage's R chunk lands while the current one is probed.
+//
+// The slot of a key inside the smem table is a multiplicative hash of the key
+// (2 instructions) rather than more bits of the partition hash: every tuple of
+// a co-partition shares the partition bits, and any function of the key that
+// spreads them works -- the result does not depend on it.
+// For each S tuple the chain is walked to its end (bag semantics); the
+// aggregation body of a match runs with the lanes converged, once per round.
+constexpr int JN_CONSUMERS = 256;
+constexpr int JN_THREADS = JN_CONSUMERS + 32;
 constexpr int JN_U = 4;
+constexpr uint32_t JN_MAXCAP = 16384;
 constexpr uint32_t JN_NIL = 0xFFFFu;
+constexpr uint32_t JN_STOP = 0xFFFFFFFFu;
 
 template <int KW, int PRW, int PSW>
 __host__ __device__ constexpr size_t join_smem_bytes(uint32_t cap, uint32_t slot_bits) {
-  return (size_t)cap * (KW + PRW) + (size_t)cap * 2 + ((size_t)4 << slot_bits) + 16;
+  return 2 * (((size_t)cap * KW + 32 + 15) / 16 * 16 + ((size_t)cap * PRW + 32 + 15) / 16 * 16)  // R ring
+         + ((size_t)cap * 2 + 15) / 16 * 16                                                        // next[]
+         + ((size_t)4 << slot_bits);                                                               // heads[]
 }
 
 struct JoinArgs {
@@ -473,148 +580,220 @@ struct JoinArgs {
   void* out_r; void* out_s; unsigned long long out_cap; unsigned long long* out_ctr;
 };
 
+struct JnStage {
+  uint32_t nr;      // R tuples in the chunk (JN_STOP = no more stages)
+  uint32_t koff;    // byte offset of element 0 inside the key buffer
+  uint32_t poff;    // byte offset of element 0 inside the payload buffer
+  uint32_t s_lo, s_hi;
+};
+
+__device__ __forceinline__ void consumer_sync() {
+  asm volatile("bar.sync 1, %0;" ::"n"(JN_CONSUMERS) : "memory");
+}
+__device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
+  asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
+}
+
+// slot of a key in the smem table: top slot_bits bits of key * odd constant
+template <int KW>
+__device__ __forceinline__ uint32_t jn_slot(typename UW<KW>::T k, uint32_t sbits) {
+  if constexpr (KW == 4) return (uint32_t)(k * 0x9E3779B1u) >> (32 - sbits);
+  else return (uint32_t)((k * 0x9E3779B97F4A7C15ull) >> (64 - sbits));
+}
+
+struct JnAcc {
+  unsigned long long cnt = 0, sr = 0, ss = 0, sx = 0;
+};
+
+template <int KW, int PRW, int PSW>
+struct JnTable {
+  const typename UW<KW>::T* k;     // R chunk keys (landing buffer)
+  const typename UW<PRW>::S* p;    // R chunk payloads
+  const uint16_t* next;
+  const uint32_t* head;
+  uint32_t sbits;
+};
+
+// Probe U S tuples per consumer thread: j = base + u*256 + tid.
+template <int KW, int PRW, int PSW, bool MAT, int U>
+__device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, PSW>& t, const JoinArgs& a, uint32_t base,
+                                               uint32_t s_hi, JnAcc& acc, uint32_t* s_wsum,
+                                               unsigned long long* s_wbase) {
+  using K = typename UW<KW>::T;
+  using PS = typename UW<PSW>::S;
+  const K* __restrict__ sk = static_cast<const K*>(a.sk);
+  const PS* __restrict__ sp = static_cast<const PS*>(a.sp);
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  K k[U];
+  PS v[U];
+  uint32_t e0[U];
+#pragma unroll
+  for (int u = 0; u < U; u++) {
+    const uint32_t j = base + u * JN_CONSUMERS + threadIdx.x;
+    if (j < s_hi) { k[u] = __ldcs(sk + j); v[u] = __ldcs(sp + j); }
+  }
+#pragma unroll
+  for (int u = 0; u < U; u++) {
+    const uint32_t j = base + u * JN_CONSUMERS + threadIdx.x;
+    e0[u] = j < s_hi ? t.head[jn_slot<KW>(k[u], t.sbits)] : JN_NIL;
+  }
+  uint32_t c[U];
+#pragma unroll
+  for (int u = 0; u < U; u++) {
+    // walk to the next match (divergent, cheap), then run the aggregation
+    // body once per round with every lane that found one (converged)
+    c[u] = 0;
+    uint32_t e = e0[u];
+    while (true) {
+      while (e != JN_NIL && t.k[e] != k[u]) e = t.next[e];
+      const bool hit = e != JN_NIL;
+      if (!__any_sync(0xffffffffu, hit)) break;
+      if (hit) {
+        const int64_t pr = (int64_t)t.p[e], ps = (int64_t)v[u];
+        c[u]++;
+        acc.sr += (unsigned long long)pr;
+        acc.ss += (unsigned long long)ps;
+        acc.sx += pair_mix(pr, ps);
+        e = t.next[e];
+      }
+    }
+    acc.cnt += c[u];
+  }
+  if constexpr (MAT) {
+    // positions in (u-major, lane-minor) order inside the warp, warps in order
+    // inside the block, one global claim per block per batch
+    uint32_t incl[U], before[U], wtot = 0;
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      incl[u] = warp_incl_scan(c[u]);
+      before[u] = wtot;
+      wtot += __shfl_sync(0xffffffffu, incl[u], 31);
+    }
+    if (lane == 0) s_wsum[warp] = wtot;
+    consumer_sync();
+    if (threadIdx.x == 0) {
+      unsigned long long run = 0;
+      for (int w = 0; w < JN_CONSUMERS / 32; w++) { s_wbase[w] = run; run += s_wsum[w]; }
+      const unsigned long long g = run ? atomicAdd(a.out_ctr, run) : 0ull;
+      for (int w = 0; w < JN_CONSUMERS / 32; w++) s_wbase[w] += g;
+    }
+    consumer_sync();
+    const unsigned long long wb = s_wbase[warp];
+    using PR = typename UW<PRW>::S;
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      if (!c[u]) continue;
+      unsigned long long pos = wb + before[u] + incl[u] - c[u];
+      for (uint32_t e = e0[u]; e != JN_NIL; e = t.next[e]) {
+        if (t.k[e] == k[u]) {
+          if (pos < a.out_cap) {
+            static_cast<PR*>(a.out_r)[pos] = t.p[e];
+            static_cast<PS*>(a.out_s)[pos] = v[u];
+          }
+          pos++;
+        }
+      }
+    }
+  }
+}
+
 template <int KW, int PRW, int PSW, bool MAT>
 __global__ void __launch_bounds__(JN_THREADS)
 k_build_probe(JoinArgs a) {
   using K = typename UW<KW>::T;
   using PR = typename UW<PRW>::S;
-  using PS = typename UW<PSW>::S;
-  extern __shared__ __align__(16) unsigned char smem[];
-  K* s_rk = reinterpret_cast<K*>(smem);
-  PR* s_rp = reinterpret_cast<PR*>(smem + (size_t)a.cap * KW);
-  uint16_t* s_next = reinterpret_cast<uint16_t*>(smem + (size_t)a.cap * (KW + PRW));
-  uint32_t* s_head = reinterpret_cast<uint32_t*>(smem + (size_t)a.cap * (KW + PRW + 2) +
-                                                  (((size_t)a.cap * 2) & 2));  // 4-B align
-  __shared__ uint32_t s_item;
-  __shared__ uint32_t s_wsum[JN_THREADS / 32];
-  __shared__ unsigned long long s_wbase[JN_THREADS / 32];
+  extern __shared__ __align__(128) unsigned char smem[];
+  const uint32_t RKB = (a.cap * KW + 32 + 15) / 16 * 16, RPB = (a.cap * PRW + 32 + 15) / 16 * 16;
+  unsigned char* ring = smem;                                           // [2][RKB | RPB]
+  uint16_t* s_next = reinterpret_cast<uint16_t*>(smem + 2 * (RKB + RPB));
+  uint32_t* s_head = reinterpret_cast<uint32_t*>(smem + 2 * (RKB + RPB) + ((size_t)a.cap * 2 + 15) / 16 * 16);
+  __shared__ JnStage s_meta[2];
+  __shared__ __align__(8) uint64_t full[2], empty[2];
+  __shared__ uint32_t s_wsum[JN_CONSUMERS / 32];
+  __shared__ unsigned long long s_wbase[JN_CONSUMERS / 32];
   __shared__ unsigned long long s_red[4][JN_THREADS / 32];
 
-  const K* __restrict__ rk = static_cast<const K*>(a.rk);
-  const PR* __restrict__ rp = static_cast<const PR*>(a.rp);
-  const K* __restrict__ sk = static_cast<const K*>(a.sk);
-  const PS* __restrict__ sp = static_cast<const PS*>(a.sp);
-  const uint32_t nslots = 1u << a.slot_bits, smask = nslots - 1;
+  const uint32_t nslots = 1u << a.slot_bits;
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  JnAcc acc;
 
-  unsigned long long cnt = 0, sr = 0, ss = 0, sx = 0;
-  uint32_t epoch = 0;  // heads with another epoch are empty
-  for (uint32_t i = threadIdx.x; i < nslots; i += JN_THREADS) s_head[i] = 0;
-  const uint32_t n_items = *a.n_items;
+  if (threadIdx.x == 0) {
+    for (int i = 0; i < 2; i++) { mbar_init(&full[i], 1); mbar_init(&empty[i], 1); }
+    asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+  }
+  __syncthreads();
 
-  while (true) {
-    __syncthreads();
-    if (threadIdx.x == 0) s_item = atomicAdd(a.item_ctr, 1u);
-    __syncthreads();
-    const uint32_t it = s_item;
-    if (it >= n_items) break;
-    const uint2 item = a.items[it];
-    const uint32_t q = item.x;
-    const uint32_t r_lo = a.bR[q], r_hi = a.bR[q + 1];
-    const uint32_t s_lo = a.bS[q] + item.y * a.slice;
-    const uint32_t s_hi = min(a.bS[q + 1], s_lo + a.slice);
-
-    for (uint32_t c_lo = r_lo; c_lo < r_hi; c_lo += a.cap) {
-      const uint32_t nr = min(a.cap, r_hi - c_lo);
-      if (++epoch == 0x10000u) {  // epoch wrap: clear the heads once
-        for (uint32_t i = threadIdx.x; i < nslots; i += JN_THREADS) s_head[i] = 0;
-        epoch = 1;
-        __syncthreads();
+  if (warp == JN_CONSUMERS / 32) {
+    // ------------------------------ producer warp ------------------------------
+    if (lane == 0) {
+      const uint64_t pol = policy_evict_first();
+      const uint32_t n_items = *a.n_items;
+      const char* rkb = static_cast<const char*>(a.rk);
+      const char* rpb = static_cast<const char*>(a.rp);
+      uint32_t stage = 0;
+      for (uint32_t it = blockIdx.x; it < n_items; it += gridDim.x) {
+        const uint2 item = a.items[it];
+        const uint32_t q = item.x;
+        const uint32_t r_lo = a.bR[q], r_hi = a.bR[q + 1];
+        const uint32_t s_lo = a.bS[q] + item.y * a.slice;
+        const uint32_t s_hi = min(a.bS[q + 1], s_lo + a.slice);
+        for (uint32_t c_lo = r_lo; c_lo < r_hi; c_lo += a.cap, stage++) {
+          const uint32_t bi = stage & 1, ph = (stage >> 1) & 1;
+          mbar_wait_backoff(&empty[bi], ph ^ 1);
+          const uint32_t nr = min(a.cap, r_hi - c_lo);
+          const uintptr_t ka = reinterpret_cast<uintptr_t>(rkb + (size_t)c_lo * KW);
+          const uintptr_t pa = reinterpret_cast<uintptr_t>(rpb + (size_t)c_lo * PRW);
+          const uintptr_t k0 = ka & ~(uintptr_t)15, k1 = (ka + (size_t)nr * KW + 15) & ~(uintptr_t)15;
+          const uintptr_t p0 = pa & ~(uintptr_t)15, p1 = (pa + (size_t)nr * PRW + 15) & ~(uintptr_t)15;
+          s_meta[bi] = JnStage{nr, (uint32_t)(ka - k0), (uint32_t)(pa - p0), s_lo, s_hi};
+          unsigned char* kbuf = ring + bi * (RKB + RPB);
+          mbar_expect_tx(&full[bi], (uint32_t)((k1 - k0) + (p1 - p0)));
+          bulk_g2s_ef(kbuf, reinterpret_cast<const void*>(k0), (uint32_t)(k1 - k0), &full[bi], pol);
+          bulk_g2s_ef(kbuf + RKB, reinterpret_cast<const void*>(p0), (uint32_t)(p1 - p0), &full[bi], pol);
+        }
       }
-      // ---- build (a11): R chunk -> smem, chained table via atomicExch
-      for (uint32_t i = threadIdx.x; i < nr; i += JN_THREADS) {
-        const K k = rk[c_lo + i];
-        s_rk[i] = k;
-        s_rp[i] = rp[c_lo + i];
-        const uint32_t slot = (uint32_t)(part_hash<KW>(k, a.ident) >> a.slot_shift) & smask;
-        const uint32_t old = atomicExch(&s_head[slot], (epoch << 16) | i);
-        s_next[i] = (old >> 16) == epoch ? (uint16_t)(old & 0xFFFFu) : (uint16_t)JN_NIL;
-      }
-      __syncthreads();
+      const uint32_t bi = stage & 1, ph = (stage >> 1) & 1;
+      mbar_wait_backoff(&empty[bi], ph ^ 1);
+      s_meta[bi].nr = JN_STOP;
+      mbar_arrive(&full[bi]);
+    }
+  } else {
+    // ------------------------------ consumer warps -----------------------------
+    for (uint32_t stage = 0;; stage++) {
+      const uint32_t bi = stage & 1, ph = (stage >> 1) & 1;
+      // reset the heads (the previous stage's probe is complete: see the
+      // barrier at the end of the loop body), then wait for the R chunk
+      for (uint32_t i = threadIdx.x * 4; i < nslots; i += JN_CONSUMERS * 4)
+        *reinterpret_cast<uint4*>(s_head + i) = make_uint4(JN_NIL, JN_NIL, JN_NIL, JN_NIL);
+      mbar_wait(&full[bi], ph);
+      const JnStage st = s_meta[bi];
+      if (st.nr == JN_STOP) break;
+      const unsigned char* kbuf = ring + bi * (RKB + RPB);
+      const K* s_rk = reinterpret_cast<const K*>(kbuf + st.koff);
+      const PR* s_rp = reinterpret_cast<const PR*>(kbuf + RKB + st.poff);
+      consumer_sync();
+      // ---- build (a11): chained table via atomicExch on the heads
+      for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
+        s_next[i] = (uint16_t)atomicExch(&s_head[jn_slot<KW>(s_rk[i], a.slot_bits)], i);
+      consumer_sync();
       // ---- probe (a12): stream the S slice
-      for (uint32_t base = s_lo; base < s_hi; base += JN_THREADS * JN_U) {
-        K k[JN_U];
-        PS v[JN_U];
-        uint32_t head[JN_U];
-#pragma unroll
-        for (int u = 0; u < JN_U; u++) {
-          const uint32_t j = base + u * JN_THREADS + threadIdx.x;
-          if (j < s_hi) { k[u] = __ldcs(sk + j); v[u] = __ldcs(sp + j); }
-        }
-#pragma unroll
-        for (int u = 0; u < JN_U; u++) {
-          const uint32_t j = base + u * JN_THREADS + threadIdx.x;
-          head[u] = JN_NIL;
-          if (j < s_hi) {
-            const uint32_t slot = (uint32_t)(part_hash<KW>(k[u], a.ident) >> a.slot_shift) & smask;
-            const uint32_t h = s_head[slot];
-            head[u] = (h >> 16) == epoch ? (h & 0xFFFFu) : JN_NIL;
-          }
-        }
-        uint32_t c[JN_U];
-#pragma unroll
-        for (int u = 0; u < JN_U; u++) {
-          // walk the chain to the next match (cheap, divergent), then run the
-          // aggregation body once per round for all lanes that found one
-          // (converged), so the checksum's 64-bit mixing is not replayed per
-          // divergent chain position
-          c[u] = 0;
-          uint32_t e = head[u];
-          while (true) {
-            while (e != JN_NIL && s_rk[e] != k[u]) e = s_next[e];
-            const bool hit = e != JN_NIL;
-            if (!__any_sync(0xffffffffu, hit)) break;
-            if (hit) {
-              const int64_t pr = (int64_t)s_rp[e], ps = (int64_t)v[u];
-              c[u]++;
-              sr += (unsigned long long)pr;
-              ss += (unsigned long long)ps;
-              sx += pair_mix(pr, ps);
-              e = s_next[e];
-            }
-          }
-          cnt += c[u];
-        }
-        if constexpr (MAT) {
-          // positions: (u-major, lane-minor) order inside the warp, warps in
-          // order inside the block, one global claim per block per batch
-          uint32_t incl[JN_U], wtot = 0, before[JN_U];
-#pragma unroll
-          for (int u = 0; u < JN_U; u++) {
-            incl[u] = warp_incl_scan(c[u]);
-            before[u] = wtot;
-            wtot += __shfl_sync(0xffffffffu, incl[u], 31);
-          }
-          if (lane == 0) s_wsum[warp] = wtot;
-          __syncthreads();
-          if (threadIdx.x == 0) {
-            unsigned long long run = 0;
-            for (int w = 0; w < JN_THREADS / 32; w++) { s_wbase[w] = run; run += s_wsum[w]; }
-            const unsigned long long g = run ? atomicAdd(a.out_ctr, run) : 0ull;
-            for (int w = 0; w < JN_THREADS / 32; w++) s_wbase[w] += g;
-          }
-          __syncthreads();
-          const unsigned long long wb = s_wbase[warp];
-#pragma unroll
-          for (int u = 0; u < JN_U; u++) {
-            if (!c[u]) continue;
-            unsigned long long pos = wb + before[u] + incl[u] - c[u];
-            for (uint32_t e = head[u]; e != JN_NIL; e = s_next[e]) {
-              if (s_rk[e] == k[u]) {
-                if (pos < a.out_cap) {
-                  static_cast<PR*>(a.out_r)[pos] = s_rp[e];
-                  static_cast<PS*>(a.out_s)[pos] = v[u];
-                }
-                pos++;
-              }
-            }
-          }
-        }
-      }
-      __syncthreads();
+      const JnTable<KW, PRW, PSW> tab{s_rk, s_rp, s_next, s_head, a.slot_bits};
+      uint32_t base = st.s_lo;
+      for (; base + JN_U * JN_CONSUMERS <= st.s_hi; base += JN_U * JN_CONSUMERS)
+        jn_probe_batch<KW, PRW, PSW, MAT, JN_U>(tab, a, base, st.s_hi, acc, s_wsum, s_wbase);
+      const uint32_t rem = st.s_hi > base ? st.s_hi - base : 0;
+      if (rem > 2 * JN_CONSUMERS)
+        jn_probe_batch<KW, PRW, PSW, MAT, 4>(tab, a, base, st.s_hi, acc, s_wsum, s_wbase);
+      else if (rem > JN_CONSUMERS)
+        jn_probe_batch<KW, PRW, PSW, MAT, 2>(tab, a, base, st.s_hi, acc, s_wsum, s_wbase);
+      else if (rem > 0)
+        jn_probe_batch<KW, PRW, PSW, MAT, 1>(tab, a, base, st.s_hi, acc, s_wsum, s_wbase);
+      consumer_sync();  // everyone is done with heads/next and ring buffer bi
+      if (threadIdx.x == 0) mbar_arrive(&empty[bi]);
     }
   }
   // ---- a13: block reduction of the four u64 partials, one atomic each
+  unsigned long long cnt = acc.cnt, sr = acc.sr, ss = acc.ss, sx = acc.sx;
 #pragma unroll
   for (int o = 16; o > 0; o >>= 1) {
     cnt += __shfl_xor_sync(0xffffffffu, cnt, o);

@@ -4,10 +4,13 @@ import csv, subprocess, sys
 for rep in sys.argv[1:]:
     out = subprocess.run(["ncu", "-i", rep, "--page", "raw", "--csv"], capture_output=True, text=True).stdout
     r = list(csv.reader(out.splitlines()))
-    h, v = r[0], r[2]
+    h, units, v = r[0], r[1], r[2]
     d = dict(zip(h, v))
+    U = dict(zip(h, units))
+    SCALE = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9, "nsecond": 1, "usecond": 1e3,
+             "msecond": 1e6, "second": 1e9}
     def g(k):
-        try: return float(d[k].replace(",", ""))
+        try: return float(d[k].replace(",", "")) * SCALE.get(U.get(k, ""), 1)
         except Exception: return float("nan")
     dur = g("gpu__time_duration.sum")
     rd, wr = g("dram__bytes_read.sum"), g("dram__bytes_write.sum")
