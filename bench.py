@@ -170,6 +170,8 @@ def main():
     ap.add_argument("--no-cpu-baseline", action="store_true")
     ap.add_argument("--no-e2e", action="store_true")
     ap.add_argument("--verify", action="store_true", help="check the result against generator provenance")
+    ap.add_argument("--bits", default="0,0", help="radix bits per pass (0 = auto; tuning only)")
+    ap.add_argument("--passes", type=int, default=0, help="radix passes (0 = auto; tuning only)")
     args = ap.parse_args()
     if args.impl == "reference":
         return run_reference(args)
@@ -206,6 +208,7 @@ def main():
     stream = torch.cuda.current_stream()
     j = RadixJoin(key_dtype=kdt, r_payload_dtype=pdt, s_payload_dtype=pdt, device=local,
                   max_r=nr_loc, max_s=ns_loc, world_size=world, rank=rank,
+                  radix_passes=args.passes, radix_bits=tuple(int(x) for x in args.bits.split(",")),
                   nccl_comm=comm, stream=stream)
     out_r = out_s = None
     if materialize:

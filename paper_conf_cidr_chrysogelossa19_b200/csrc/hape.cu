@@ -20,6 +20,7 @@
 #include <cstdlib>
 #include <cstring>
 #include <string>
+#include <type_traits>
 #include <vector>
 
 #include "hape.h"
@@ -61,10 +62,10 @@ struct hape_join {
   uint32_t launches = 0;
   // workspace
   DevBuf stage[4];        // host-input staging: R key, R pay, S key, S pay
-  DevBuf ping[4];         // pass-1 output
-  DevBuf pong[4];         // pass-2 output
-  DevBuf send[4];         // G>1 device-partition output
-  DevBuf recv[4];         // G>1 exchange receive buffers
+  DevBuf ping[2];         // pass-1 output tuples (R, S)
+  DevBuf pong[2];         // pass-2 output tuples
+  DevBuf send[2];         // G>1 device-partition output tuples
+  DevBuf recv[2];         // G>1 exchange receive buffers
   DevBuf outst[2];        // host-output staging
   DevBuf small;           // histograms, bounds, work list, counters
   unsigned long long* h_res = nullptr;  // pinned: acc[4], out_ctr, (n_items | item_ctr)
@@ -220,23 +221,36 @@ static hape_status make_plan(const hape_join* h, uint64_t n_r, uint64_t n_s, hap
 // ---------------------------------------------------------------------------
 // kernel launchers (dtype dispatch)
 // ---------------------------------------------------------------------------
-struct Col {
-  const void* k;
-  const void* p;
+// A relation as a partitioning pass sees it: SoA columns or AoS tuples.
+struct Src {
+  PartIn in;
+  bool aos;
   uint32_t n;
   int pw;
 };
 
-static hape_status launch_hist(hape_join* h, int kw, const void* key, SegMap m, BitField bf, uint32_t P,
-                               uint32_t* hist, uint32_t* rowsum) {
+static size_t tup_bytes(int kw, int pw) { return (kw + pw) <= 8 ? 8 : 16; }
+
+template <int KW, int PW, bool AOS>
+static void hist_t(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* hist, uint32_t* rowsum) {
   const unsigned grid = m.nseg * m.cps;
-  const size_t smem = (size_t)P * 4;
-  const int ident = h->cfg.part_fn == HAPE_PART_IDENTITY;
-  if (grid == 0) return HAPE_OK;
-  if (kw == 4)
-    k_hist<4><<<grid, HIST_THREADS, smem, h->stream>>>((const uint32_t*)key, m, bf, ident, P, hist, rowsum);
-  else
-    k_hist<8><<<grid, HIST_THREADS, smem, h->stream>>>((const uint64_t*)key, m, bf, ident, P, hist, rowsum);
+  k_hist<KW, PW, AOS><<<grid, HIST_THREADS, (size_t)P * 4, h->stream>>>(s.in, m, bf, h->cfg.part_fn == HAPE_PART_IDENTITY,
+                                                                        P, hist, rowsum);
+}
+
+static hape_status launch_hist(hape_join* h, int kw, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* hist,
+                               uint32_t* rowsum) {
+  if (m.nseg * m.cps == 0) return HAPE_OK;
+  const int pw = s.pw;
+  if (s.aos) {
+    if (kw == 4 && pw == 4) hist_t<4, 4, true>(h, s, m, bf, P, hist, rowsum);
+    else if (kw == 4) hist_t<4, 8, true>(h, s, m, bf, P, hist, rowsum);
+    else if (pw == 4) hist_t<8, 4, true>(h, s, m, bf, P, hist, rowsum);
+    else hist_t<8, 8, true>(h, s, m, bf, P, hist, rowsum);
+  } else {
+    if (kw == 4) hist_t<4, 4, false>(h, s, m, bf, P, hist, rowsum);  // keys only: PW irrelevant
+    else hist_t<8, 8, false>(h, s, m, bf, P, hist, rowsum);
+  }
   CK_LAUNCH(h);
   return HAPE_OK;
 }
@@ -251,36 +265,60 @@ static hape_status launch_scan(hape_join* h, SegMap m, uint32_t P, uint32_t* his
   return HAPE_OK;
 }
 
-template <int KW, int PW>
-static hape_status launch_scatter_t(hape_join* h, const Col& in, SegMap m, BitField bf, uint32_t P,
-                                    const uint32_t* offs, void* ok, void* op) {
-  const size_t smem = scatter_smem_bytes<KW, PW>(P);
+template <int KW, int PW, bool AOS, class C>
+static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, const uint32_t* offs,
+                             void* out) {
+  const size_t smem = ScLayout<KW, PW, AOS, C>::bytes(P);
   static bool attr_set = false;
   if (!attr_set) {
-    CK(h, cudaFuncSetAttribute(k_scatter<KW, PW>, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024));
+    CK(h, cudaFuncSetAttribute(k_scatter<KW, PW, AOS, C>, cudaFuncAttributeMaxDynamicSharedMemorySize, 220 * 1024));
     attr_set = true;
   }
   const unsigned grid = m.nseg * m.cps;
   if (grid == 0) return HAPE_OK;
-  k_scatter<KW, PW><<<grid, SC_THREADS, smem, h->stream>>>(
-      (const typename UW<KW>::T*)in.k, (const typename UW<PW>::T*)in.p, m, bf,
-      h->cfg.part_fn == HAPE_PART_IDENTITY, P, offs, (typename UW<KW>::T*)ok, (typename UW<PW>::T*)op);
+  k_scatter<KW, PW, AOS, C><<<grid, C::NT, smem, h->stream>>>(s.in, m, bf, h->cfg.part_fn == HAPE_PART_IDENTITY, P,
+                                                             offs, static_cast<Tup<KW, PW>*>(out));
   CK_LAUNCH(h);
   return HAPE_OK;
 }
 
-static hape_status launch_scatter(hape_join* h, int kw, const Col& in, SegMap m, BitField bf, uint32_t P,
-                                  const uint32_t* offs, void* ok, void* op) {
-  if (kw == 4 && in.pw == 4) return launch_scatter_t<4, 4>(h, in, m, bf, P, offs, ok, op);
-  if (kw == 4 && in.pw == 8) return launch_scatter_t<4, 8>(h, in, m, bf, P, offs, ok, op);
-  if (kw == 8 && in.pw == 4) return launch_scatter_t<8, 4>(h, in, m, bf, P, offs, ok, op);
-  return launch_scatter_t<8, 8>(h, in, m, bf, P, offs, ok, op);
+// scatter shape per tuple width; HAPE_SC selects alternatives (tuning only)
+template <int KW, int PW, bool AOS>
+static hape_status scatter_v(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, const uint32_t* offs,
+                             void* out) {
+  static int v = [] { const char* e = getenv("HAPE_SC"); return e ? atoi(e) : -1; }();
+  if constexpr (KW + PW <= 8) {
+    switch (v) {
+      case 1: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 1>>(h, s, m, bf, P, offs, out);
+      case 2: return scatter_t<KW, PW, AOS, ScCfg<256, 16, 2>>(h, s, m, bf, P, offs, out);
+      case 3: return scatter_t<KW, PW, AOS, ScCfg<1024, 8, 1>>(h, s, m, bf, P, offs, out);
+      case 4: return scatter_t<KW, PW, AOS, ScCfg<256, 8, 2>>(h, s, m, bf, P, offs, out);
+      default: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 2>>(h, s, m, bf, P, offs, out);
+    }
+  } else {
+    switch (v) {
+      case 1: return scatter_t<KW, PW, AOS, ScCfg<512, 4, 2>>(h, s, m, bf, P, offs, out);
+      default: return scatter_t<KW, PW, AOS, ScCfg<256, 8, 2>>(h, s, m, bf, P, offs, out);
+    }
+  }
+}
+
+static hape_status launch_scatter(hape_join* h, int kw, const Src& s, SegMap m, BitField bf, uint32_t P,
+                                  const uint32_t* offs, void* out) {
+  const int pw = s.pw;
+#define HAPE_SC_DISPATCH(AOS)                                                 \
+  if (kw == 4 && pw == 4) return scatter_v<4, 4, AOS>(h, s, m, bf, P, offs, out); \
+  if (kw == 4) return scatter_v<4, 8, AOS>(h, s, m, bf, P, offs, out);            \
+  if (pw == 4) return scatter_v<8, 4, AOS>(h, s, m, bf, P, offs, out);            \
+  return scatter_v<8, 8, AOS>(h, s, m, bf, P, offs, out);
+  if (s.aos) { HAPE_SC_DISPATCH(true) } else { HAPE_SC_DISPATCH(false) }
+#undef HAPE_SC_DISPATCH
 }
 
 template <int KW, int PRW, int PSW, bool MAT>
 static hape_status launch_join_t(hape_join* h, const JoinArgs& a, uint32_t* ctas_out) {
   auto kern = k_build_probe<KW, PRW, PSW, MAT>;
-  const size_t smem = join_smem_bytes<KW, PRW, PSW>(a.cap, a.slot_bits);
+  const size_t smem = join_smem_bytes<KW, PRW>(a.cap, a.slot_bits);
   static bool attr_set = false;
   if (!attr_set) {
     CK(h, cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024));
@@ -309,6 +347,17 @@ static hape_status launch_join(hape_join* h, int kw, int prw, int psw, const Joi
   }
   if (prw == 4) return psw == 4 ? launch_join_m<8, 4, 4>(h, a, mat, ctas) : launch_join_m<8, 4, 8>(h, a, mat, ctas);
   return psw == 4 ? launch_join_m<8, 8, 4>(h, a, mat, ctas) : launch_join_m<8, 8, 8>(h, a, mat, ctas);
+}
+
+static hape_status launch_unpack(hape_join* h, int kw, int pw, const void* t, uint32_t n, void* k, void* p) {
+  if (!n) return HAPE_OK;
+  const unsigned grid = std::min<unsigned>((n + 255) / 256, 4096);
+  if (kw == 4 && pw == 4) k_unpack<4, 4><<<grid, 256, 0, h->stream>>>((const Tup<4, 4>*)t, n, (uint32_t*)k, (uint32_t*)p);
+  else if (kw == 4) k_unpack<4, 8><<<grid, 256, 0, h->stream>>>((const Tup<4, 8>*)t, n, (uint32_t*)k, (uint64_t*)p);
+  else if (pw == 4) k_unpack<8, 4><<<grid, 256, 0, h->stream>>>((const Tup<8, 4>*)t, n, (uint64_t*)k, (uint32_t*)p);
+  else k_unpack<8, 8><<<grid, 256, 0, h->stream>>>((const Tup<8, 8>*)t, n, (uint64_t*)k, (uint64_t*)p);
+  CK_LAUNCH(h);
+  return HAPE_OK;
 }
 
 // ---------------------------------------------------------------------------
@@ -374,17 +423,16 @@ static T* at(hape_join* h, size_t off) {
   return reinterpret_cast<T*>(static_cast<char*>(h->small.p) + off);
 }
 
-// Radix passes over one relation: in -> (ping, pong) -> final columns + bounds.
-// Launches are grouped by stage across both relations by the caller.
+// Radix passes over one relation: in -> ping (AoS) -> pong (AoS) -> bounds.
+// Launches are grouped by stage across both relations.
 struct PassIO {
-  Col in;                      // pass-1 input
-  void* p1k; void* p1p;        // pass-1 output
-  void* p2k; void* p2p;        // pass-2 output
+  Src in;       // pass-1 input
+  void* p1;     // pass-1 output tuples
+  void* p2;     // pass-2 output tuples
 };
 
 static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const CallLayout& L, PassIO io[2],
-                                        int nside, const void** fin_k, const void** fin_p,
-                                        const uint32_t** fin_bounds) {
+                                        int nside, const void** fin, const uint32_t** fin_bounds) {
   const int kw = key_width(h->cfg);
   const uint32_t P1 = 1u << pl.bits[0], P2 = 1u << pl.bits[1];
   const BitField bf1{0u, P1 - 1}, bf2{pl.bits[0], P2 - 1};
@@ -395,35 +443,32 @@ static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const
   }
   mark(h, HAPE_STAGE_HIST1);
   for (int s = 0; s < nside; s++)
-    CKS(launch_hist(h, kw, io[s].in.k, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1),
-                    at<uint32_t>(h, L.side[s].rowsum1)));
+    CKS(launch_hist(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1)));
   mark(h, HAPE_STAGE_SCAN1);
   for (int s = 0; s < nside; s++)
     CKS(launch_scan(h, m1[s], P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1),
                     at<uint32_t>(h, L.side[s].bounds1)));
   mark(h, HAPE_STAGE_SCATTER1);
   for (int s = 0; s < nside; s++)
-    CKS(launch_scatter(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), io[s].p1k, io[s].p1p));
+    CKS(launch_scatter(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), io[s].p1));
   for (int s = 0; s < nside; s++) {
-    fin_k[s] = io[s].p1k;
-    fin_p[s] = io[s].p1p;
+    fin[s] = io[s].p1;
     fin_bounds[s] = at<uint32_t>(h, L.side[s].bounds1);
   }
   if (pl.passes == 2) {
+    Src s2[2];
+    for (int s = 0; s < nside; s++) s2[s] = Src{PartIn{nullptr, nullptr, io[s].p1}, true, io[s].in.n, io[s].in.pw};
     mark(h, HAPE_STAGE_HIST2);
     for (int s = 0; s < nside; s++)
-      CKS(launch_hist(h, kw, io[s].p1k, m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2),
-                      at<uint32_t>(h, L.side[s].rowsum2)));
+      CKS(launch_hist(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), at<uint32_t>(h, L.side[s].rowsum2)));
     mark(h, HAPE_STAGE_SCAN2);
     for (int s = 0; s < nside; s++)
       CKS(launch_scan(h, m2[s], P2, at<uint32_t>(h, L.side[s].hist2), at<uint32_t>(h, L.side[s].rowsum2),
                       at<uint32_t>(h, L.side[s].bounds2)));
     mark(h, HAPE_STAGE_SCATTER2);
     for (int s = 0; s < nside; s++) {
-      Col c2{io[s].p1k, io[s].p1p, io[s].in.n, io[s].in.pw};
-      CKS(launch_scatter(h, kw, c2, m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), io[s].p2k, io[s].p2p));
-      fin_k[s] = io[s].p2k;
-      fin_p[s] = io[s].p2p;
+      CKS(launch_scatter(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), io[s].p2));
+      fin[s] = io[s].p2;
       fin_bounds[s] = at<uint32_t>(h, L.side[s].bounds2);
     }
   }
@@ -445,20 +490,19 @@ static hape_status check_rel(hape_join* h, const hape_relation* r, int kw, int p
 }
 
 static hape_status stage_in(hape_join* h, const hape_relation* r, int kw, int pw, DevBuf& bk, DevBuf& bp,
-                            Col* out) {
+                            Src* out) {
   out->n = (uint32_t)r->n;
   out->pw = pw;
+  out->aos = false;
   if (r->mem == HAPE_MEM_DEVICE || r->n == 0) {
-    out->k = r->key;
-    out->p = r->payload;
+    out->in = PartIn{r->key, r->payload, nullptr};
     return HAPE_OK;
   }
   CKS(ensure(h, bk, r->n * kw));
   CKS(ensure(h, bp, r->n * pw));
   CK(h, cudaMemcpyAsync(bk.p, r->key, r->n * kw, cudaMemcpyHostToDevice, h->stream));
   CK(h, cudaMemcpyAsync(bp.p, r->payload, r->n * pw, cudaMemcpyHostToDevice, h->stream));
-  out->k = bk.p;
-  out->p = bp.p;
+  out->in = PartIn{bk.p, bp.p, nullptr};
   return HAPE_OK;
 }
 
@@ -478,7 +522,7 @@ extern "C" hape_status hape_exchange_plan(int world_size, int rank, const uint64
   return HAPE_OK;
 }
 
-static hape_status exchange(hape_join* h, Col in[2], Col out[2]) {
+static hape_status exchange(hape_join* h, Src in[2], Src out[2]) {
   const int G = h->cfg.world_size, me = h->cfg.rank;
   const int kw = key_width(h->cfg);
   const uint32_t g = ceil_log2_u64((uint64_t)G);
@@ -499,16 +543,17 @@ static hape_status exchange(hape_join* h, Col in[2], Col out[2]) {
   CK(h, cudaMemsetAsync(at<char>(h, rs_off[0]), 0, (size_t)G * 4, h->stream));
   CK(h, cudaMemsetAsync(at<char>(h, rs_off[1]), 0, (size_t)G * 4, h->stream));
   mark(h, HAPE_STAGE_DEVPART);
+  size_t tb[2];
   for (int s = 0; s < 2; s++) {
-    CKS(ensure(h, h->send[2 * s], (size_t)in[s].n * kw + 16));
-    CKS(ensure(h, h->send[2 * s + 1], (size_t)in[s].n * in[s].pw + 16));
+    tb[s] = tup_bytes(kw, in[s].pw);
+    CKS(ensure(h, h->send[s], (size_t)in[s].n * tb[s] + 16));
     SegMap m{nullptr, 1u, cps[s], in[s].n};
     uint32_t* hist = at<uint32_t>(h, hist_off[s]);
     uint32_t* rs = at<uint32_t>(h, rs_off[s]);
     uint32_t* bl = at<uint32_t>(h, bl_off) + s * (G + 1);
-    CKS(launch_hist(h, kw, in[s].k, m, bf, (uint32_t)G, hist, rs));
+    CKS(launch_hist(h, kw, in[s], m, bf, (uint32_t)G, hist, rs));
     CKS(launch_scan(h, m, (uint32_t)G, hist, rs, bl));
-    CKS(launch_scatter(h, kw, in[s], m, bf, (uint32_t)G, hist, h->send[2 * s].p, h->send[2 * s + 1].p));
+    CKS(launch_scatter(h, kw, in[s], m, bf, (uint32_t)G, hist, h->send[s].p));
   }
   mark(h, HAPE_STAGE_EXCHANGE);
   // count exchange: all-gather every rank's destination bounds
@@ -531,20 +576,17 @@ static hape_status exchange(hape_join* h, Col in[2], Col out[2]) {
     uint64_t rtot = 0;
     hape_exchange_plan(G, me, counts.data(), soff.data(), roff.data(), &rtot);
     if (rtot >= 0xFFFFFFFFull) return fail(h, HAPE_ERR_UNSUPPORTED, "received %llu tuples >= 2^32", (unsigned long long)rtot);
-    const size_t w[2] = {(size_t)kw, (size_t)in[s].pw};
-    for (int c = 0; c < 2; c++) CKS(ensure(h, h->recv[2 * s + c], rtot * w[c] + 16));
+    CKS(ensure(h, h->recv[s], rtot * tb[s] + 16));
+    const char* sb = static_cast<const char*>(h->send[s].p);
+    char* rb = static_cast<char*>(h->recv[s].p);
     CKN(h, ncclGroupStart());
-    for (int c = 0; c < 2; c++) {
-      const char* sb = static_cast<const char*>(h->send[2 * s + c].p);
-      char* rb = static_cast<char*>(h->recv[2 * s + c].p);
-      for (int p = 0; p < G; p++) {
-        const uint64_t sc = counts[(size_t)me * G + p], rc = counts[(size_t)p * G + me];
-        if (sc) CKN(h, ncclSend(sb + soff[p] * w[c], sc * w[c], ncclUint8, p, h->comm, h->stream));
-        if (rc) CKN(h, ncclRecv(rb + roff[p] * w[c], rc * w[c], ncclUint8, p, h->comm, h->stream));
-      }
+    for (int p = 0; p < G; p++) {
+      const uint64_t sc = counts[(size_t)me * G + p], rc = counts[(size_t)p * G + me];
+      if (sc) CKN(h, ncclSend(sb + soff[p] * tb[s], sc * tb[s], ncclUint8, p, h->comm, h->stream));
+      if (rc) CKN(h, ncclRecv(rb + roff[p] * tb[s], rc * tb[s], ncclUint8, p, h->comm, h->stream));
     }
     CKN(h, ncclGroupEnd());
-    out[s] = Col{h->recv[2 * s].p, h->recv[2 * s + 1].p, (uint32_t)rtot, in[s].pw};
+    out[s] = Src{PartIn{nullptr, nullptr, h->recv[s].p}, true, (uint32_t)rtot, in[s].pw};
   }
   return HAPE_OK;
 }
@@ -571,10 +613,10 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
 
   mark(h, HAPE_STAGE_TOTAL);
   mark(h, HAPE_STAGE_H2D);
-  Col in[2];
+  Src in[2];
   CKS(stage_in(h, R, kw, prw, h->stage[0], h->stage[1], &in[0]));
   CKS(stage_in(h, S, kw, psw, h->stage[2], h->stage[3], &in[1]));
-  Col loc[2] = {in[0], in[1]};
+  Src loc[2] = {in[0], in[1]};
   if (world > 1) CKS(exchange(h, in, loc));
 
   hape_plan pl;
@@ -585,12 +627,8 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   const uint64_t n_loc[2] = {loc[0].n, loc[1].n};
   const int pw[2] = {prw, psw};
   for (int s = 0; s < 2; s++) {
-    CKS(ensure(h, h->ping[2 * s], n_loc[s] * kw + 16));
-    CKS(ensure(h, h->ping[2 * s + 1], n_loc[s] * pw[s] + 16));
-    if (pl.passes == 2) {
-      CKS(ensure(h, h->pong[2 * s], n_loc[s] * kw + 16));
-      CKS(ensure(h, h->pong[2 * s + 1], n_loc[s] * pw[s] + 16));
-    }
+    CKS(ensure(h, h->ping[s], n_loc[s] * tup_bytes(kw, pw[s]) + 16));
+    if (pl.passes == 2) CKS(ensure(h, h->pong[s], n_loc[s] * tup_bytes(kw, pw[s]) + 16));
   }
   void* mat_r = nullptr;
   void* mat_s = nullptr;
@@ -607,15 +645,13 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   CK(h, cudaMemsetAsync(at<char>(h, L.zero_lo), 0, L.zero_hi - L.zero_lo, h->stream));
 
   PassIO io[2];
-  for (int s = 0; s < 2; s++)
-    io[s] = PassIO{loc[s], h->ping[2 * s].p, h->ping[2 * s + 1].p, h->pong[2 * s].p, h->pong[2 * s + 1].p};
-  const void* fk[2];
-  const void* fp[2];
+  for (int s = 0; s < 2; s++) io[s] = PassIO{loc[s], h->ping[s].p, h->pong[s].p};
+  const void* ft[2];
   const uint32_t* fb[2];
-  CKS(run_partition_stages(h, pl, L, io, 2, fk, fp, fb));
+  CKS(run_partition_stages(h, pl, L, io, 2, ft, fb));
 
   const uint32_t Q = 1u << (pl.bits[0] + (pl.passes == 2 ? pl.bits[1] : 0));
-  uint32_t* ctrs = at<uint32_t>(h, L.ctrs);  // [0] n_items, [1] item_ctr
+  uint32_t* ctrs = at<uint32_t>(h, L.ctrs);  // [0] n_items
   mark(h, HAPE_STAGE_WORKLIST);
   k_worklist<<<(Q + WL_THREADS - 1) / WL_THREADS, WL_THREADS, 0, h->stream>>>(fb[0], fb[1], Q, pl.probe_slice,
                                                                               at<uint2>(h, L.items), ctrs);
@@ -623,11 +659,10 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
 
   mark(h, HAPE_STAGE_BUILD_PROBE);
   JoinArgs ja{};
-  ja.rk = fk[0]; ja.rp = fp[0]; ja.sk = fk[1]; ja.sp = fp[1];
+  ja.rt = ft[0]; ja.st = ft[1];
   ja.bR = fb[0]; ja.bS = fb[1];
-  ja.items = at<uint2>(h, L.items); ja.n_items = ctrs; ja.item_ctr = ctrs + 1;
-  ja.cap = pl.build_cap; ja.slice = pl.probe_slice; ja.slot_shift = pl.slot_shift; ja.slot_bits = pl.slot_bits;
-  ja.ident = c.part_fn == HAPE_PART_IDENTITY;
+  ja.items = at<uint2>(h, L.items); ja.n_items = ctrs;
+  ja.cap = pl.build_cap; ja.slice = pl.probe_slice; ja.slot_bits = pl.slot_bits;
   ja.acc = at<unsigned long long>(h, L.acc);
   ja.out_r = mat_r; ja.out_s = mat_s; ja.out_cap = mat ? out->capacity : 0;
   ja.out_ctr = at<unsigned long long>(h, L.out_ctr);
@@ -773,9 +808,11 @@ hape_status hape_join_destroy(hape_join* h) {
   if (!h) return HAPE_OK;
   cudaSetDevice(h->dev);
   if (h->stream) cudaStreamSynchronize(h->stream);
-  DevBuf* groups[] = {h->stage, h->ping, h->pong, h->send, h->recv};
+  for (auto& b : h->stage)
+    if (b.p) cudaFree(b.p);
+  DevBuf* groups[] = {h->ping, h->pong, h->send, h->recv};
   for (DevBuf* g : groups)
-    for (int i = 0; i < 4; i++)
+    for (int i = 0; i < 2; i++)
       if (g[i].p) cudaFree(g[i].p);
   for (auto& b : h->outst)
     if (b.p) cudaFree(b.p);
@@ -823,26 +860,20 @@ hape_status hape_debug_partition(hape_join* h, const hape_relation* rel, int is_
   if (pl.passes < 1 || pl.passes > 2 || pl.bits[0] > kMaxBitsPerPass || pl.bits[1] > kMaxBitsPerPass)
     return fail(h, HAPE_ERR_INVALID_ARG, "invalid plan");
   h->launches = 0;
-  Col in;
+  Src in;
   CKS(stage_in(h, rel, kw, pw, h->stage[0], h->stage[1], &in));
   const CallLayout L = layout_for(h, pl, rel->n, rel->n);
   CKS(ensure(h, h->small, L.total));
-  CKS(ensure(h, h->ping[0], rel->n * kw + 16));
-  CKS(ensure(h, h->ping[1], rel->n * pw + 16));
-  CKS(ensure(h, h->pong[0], rel->n * kw + 16));
-  CKS(ensure(h, h->pong[1], rel->n * pw + 16));
+  CKS(ensure(h, h->ping[0], rel->n * tup_bytes(kw, pw) + 16));
+  CKS(ensure(h, h->pong[0], rel->n * tup_bytes(kw, pw) + 16));
   CK(h, cudaMemsetAsync(at<char>(h, L.zero_lo), 0, L.zero_hi - L.zero_lo, h->stream));
   PassIO io[2];
-  io[0] = PassIO{in, h->ping[0].p, h->ping[1].p, h->pong[0].p, h->pong[1].p};
-  const void* fk[2];
-  const void* fp[2];
+  io[0] = PassIO{in, h->ping[0].p, h->pong[0].p};
+  const void* ft[2];
   const uint32_t* fb[2];
-  CKS(run_partition_stages(h, pl, L, io, 1, fk, fp, fb));
+  CKS(run_partition_stages(h, pl, L, io, 1, ft, fb));
   const uint64_t Q = 1ull << (pl.bits[0] + (pl.passes == 2 ? pl.bits[1] : 0));
-  if (rel->n) {
-    CK(h, cudaMemcpyAsync(out_keys, fk[0], rel->n * kw, cudaMemcpyDeviceToDevice, h->stream));
-    CK(h, cudaMemcpyAsync(out_payloads, fp[0], rel->n * pw, cudaMemcpyDeviceToDevice, h->stream));
-  }
+  CKS(launch_unpack(h, kw, pw, ft[0], (uint32_t)rel->n, out_keys, out_payloads));
   CK(h, cudaMemcpyAsync(out_bounds, fb[0], (Q + 1) * 4, cudaMemcpyDeviceToDevice, h->stream));
   CK(h, cudaStreamSynchronize(h->stream));
   if (plan_out) *plan_out = pl;

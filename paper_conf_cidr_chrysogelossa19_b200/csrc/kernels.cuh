@@ -17,11 +17,13 @@
 //   * the micro-benchmark consumer: count and sum over each payload column
 //     (P789-793), fused into the probe epilogue.
 //
-// Data layout in HBM: structure-of-arrays everywhere (caller columns and the
-// ping-pong workspace), uint32 tuple indices (n < 2^32 per relation per rank).
+// Data layout in HBM: caller columns are structure-of-arrays; the ping-pong
+// workspace written by the radix passes holds (key, payload) tuples (AoS,
+// struct Tup); uint32 tuple indices (n < 2^32 per relation per rank).
 // Nothing here is a dense contraction: no tensor cores.
 #pragma once
 #include <cstdint>
+#include <type_traits>
 #include <cuda_runtime.h>
 
 namespace hape {
@@ -166,36 +168,138 @@ __device__ __forceinline__ uint32_t block_exscan_strided(uint32_t* a, uint32_t n
 }
 
 // --------------------------------------------------------------------------
+// Workspace tuple: the radix passes write (key, payload) pairs (AoS), so a
+// bucket run of r tuples is one contiguous r*sizeof(Tup)-byte store run
+// instead of two half-length column runs -- the write-combining the paper's
+// scratchpad reorder is for (P579-589) then works on twice the bytes.
+// --------------------------------------------------------------------------
+template <int KW, int PW>
+struct alignas((KW + PW) <= 8 ? 8 : 16) Tup {
+  typename UW<KW>::T k;
+  typename UW<PW>::T v;
+};
+
+// streaming (evict-first) load of one tuple
+template <int KW, int PW>
+__device__ __forceinline__ Tup<KW, PW> ldcs_tup(const Tup<KW, PW>* p) {
+  Tup<KW, PW> x;
+  if constexpr (sizeof(Tup<KW, PW>) == 8) {
+    const uint2 w = __ldcs(reinterpret_cast<const uint2*>(p));
+    x = *reinterpret_cast<const Tup<KW, PW>*>(&w);
+  } else {
+    const uint4 w = __ldcs(reinterpret_cast<const uint4*>(p));
+    x = *reinterpret_cast<const Tup<KW, PW>*>(&w);
+  }
+  return x;
+}
+
+// Input of a partitioning pass: caller SoA columns (pass 1) or workspace AoS
+// tuples (pass 2, and pass 1 after the multi-GPU exchange).
+struct PartIn {
+  const void* k;   // SoA keys   (AOS = false)
+  const void* p;   // SoA payloads
+  const void* t;   // AoS tuples (AOS = true)
+};
+
+__device__ __forceinline__ uint32_t smem_u32(const void* p) {
+  return static_cast<uint32_t>(__cvta_generic_to_shared(p));
+}
+__device__ __forceinline__ void mbar_init(uint64_t* bar, uint32_t count) {
+  asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count));
+}
+__device__ __forceinline__ void mbar_expect_tx(uint64_t* bar, uint32_t bytes) {
+  asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes)
+               : "memory");
+}
+__device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
+  asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
+}
+__device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t phase) {
+  asm volatile(
+      "{\n .reg .pred p;\n WAIT_%=:\n"
+      " mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n"
+      " @!p bra WAIT_%=;\n}\n" ::"r"(smem_u32(bar)),
+      "r"(phase)
+      : "memory");
+}
+// producer-side wait: back off between polls so a warp that is far ahead
+// does not steal issue slots from the consumers
+__device__ __forceinline__ void mbar_wait_backoff(uint64_t* bar, uint32_t phase) {
+  uint32_t ok = 0;
+  while (true) {
+    asm volatile(
+        "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n selp.u32 %0, 1, 0, p;\n}\n"
+        : "=r"(ok)
+        : "r"(smem_u32(bar)), "r"(phase)
+        : "memory");
+    if (ok) return;
+    __nanosleep(256);
+  }
+}
+__device__ __forceinline__ uint64_t policy_evict_first() {
+  uint64_t pol;
+  asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(pol));
+  return pol;
+}
+// 1-D bulk copy global -> shared (TMA engine), completion on an mbarrier,
+// streamed-once data marked evict-first in L2
+__device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes, uint64_t* bar,
+                                         uint64_t pol) {
+  asm volatile(
+      "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.L2::cache_hint [%0], [%1], %2, [%3], %4;" ::"r"(
+          smem_u32(dst)),
+      "l"(src), "r"(bytes), "r"(smem_u32(bar)), "l"(pol)
+      : "memory");
+}
+// copy [src, src + bytes) rounded out to 16-byte boundaries; returns the
+// byte offset of src inside the destination buffer
+__device__ __forceinline__ uint32_t bulk_g2s_any(void* dst, const void* src, size_t bytes, uint64_t* bar,
+                                                 uint64_t pol, uint32_t* tx) {
+  const uintptr_t a = reinterpret_cast<uintptr_t>(src);
+  const uintptr_t a0 = a & ~(uintptr_t)15, a1 = (a + bytes + 15) & ~(uintptr_t)15;
+  bulk_g2s(dst, reinterpret_cast<const void*>(a0), (uint32_t)(a1 - a0), bar, pol);
+  *tx += (uint32_t)(a1 - a0);
+  return (uint32_t)(a - a0);
+}
+
+// --------------------------------------------------------------------------
 // a6: radix histogram of one pass.  One contiguous chunk per CTA; keys only
-// (w_k bytes per tuple); shared-memory counters (P166-168: "use shared memory
-// to store histograms").  Output hist[(seg*P + p)*cps + j] (partition-major
-// inside each segment, so the segment's exclusive scan IS the offsets) and
-// the per-row totals rowsum[seg*P + p].
+// (w_k bytes per tuple from SoA input; the whole tuple from AoS input);
+// shared-memory counters (P166-168: "use shared memory to store histograms").
+// Output hist[(seg*P + p)*cps + j] (partition-major inside each segment, so
+// the segment's exclusive scan IS the offsets) and the row totals
+// rowsum[seg*P + p].  16-byte vector loads, 4 in flight per thread.
 // --------------------------------------------------------------------------
 constexpr int HIST_THREADS = 512;
-constexpr int HIST_VEC = 4;  // 16-byte loads in flight per thread per iteration
+constexpr int HIST_VEC = 4;
 
-template <int KW>
+template <int KW, int PW, bool AOS>
 __global__ void __launch_bounds__(HIST_THREADS)
-k_hist(const typename UW<KW>::T* __restrict__ key, SegMap m, BitField bf, int ident, uint32_t P,
-       uint32_t* __restrict__ hist, uint32_t* __restrict__ rowsum) {
+k_hist(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, uint32_t* __restrict__ hist,
+       uint32_t* __restrict__ rowsum) {
   extern __shared__ uint32_t sh_cnt[];
   using K = typename UW<KW>::T;
-  constexpr int PER = 16 / KW;  // keys per 16-byte vector
+  using E = typename std::conditional<AOS, Tup<KW, PW>, K>::type;  // element read
+  constexpr int ES = sizeof(E);
+  constexpr int PER = 16 / ES;  // elements per 16-byte vector
+  const E* __restrict__ base = static_cast<const E*>(AOS ? in.t : in.k);
+  auto key_of = [](const E& e) -> K {
+    if constexpr (AOS) return e.k;
+    else return e;
+  };
   for (uint32_t i = threadIdx.x; i < P; i += HIST_THREADS) sh_cnt[i] = 0;
   __syncthreads();
   uint32_t seg, j, lo, hi;
   seg_chunk(m, blockIdx.x, seg, j, lo, hi);
-  // scalar head up to a 16-byte boundary, 16-byte vector body, scalar tail
   uint32_t vlo = lo;
-  while (vlo < hi && (reinterpret_cast<uintptr_t>(key + vlo) & 15)) vlo++;
+  while (vlo < hi && (reinterpret_cast<uintptr_t>(base + vlo) & 15)) vlo++;
   const uint32_t nvec = (hi - vlo) / PER;
   const uint32_t vhi = vlo + nvec * PER;
   for (uint32_t i = lo + threadIdx.x; i < vlo; i += HIST_THREADS)
-    atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(key[i], ident), bf)], 1u);
+    atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(key_of(base[i]), ident), bf)], 1u);
   for (uint32_t i = vhi + threadIdx.x; i < hi; i += HIST_THREADS)
-    atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(key[i], ident), bf)], 1u);
-  const uint4* __restrict__ vk = reinterpret_cast<const uint4*>(key + vlo);
+    atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(key_of(base[i]), ident), bf)], 1u);
+  const uint4* __restrict__ vk = reinterpret_cast<const uint4*>(base + vlo);
   uint32_t v = threadIdx.x;
   for (; v + (HIST_VEC - 1) * HIST_THREADS < nvec; v += HIST_VEC * HIST_THREADS) {
     uint4 w[HIST_VEC];
@@ -203,16 +307,16 @@ k_hist(const typename UW<KW>::T* __restrict__ key, SegMap m, BitField bf, int id
     for (int u = 0; u < HIST_VEC; u++) w[u] = __ldcs(vk + v + u * HIST_THREADS);
 #pragma unroll
     for (int u = 0; u < HIST_VEC; u++) {
-      const K* kk = reinterpret_cast<const K*>(&w[u]);
+      const E* ee = reinterpret_cast<const E*>(&w[u]);
 #pragma unroll
-      for (int e = 0; e < PER; e++) atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(kk[e], ident), bf)], 1u);
+      for (int e = 0; e < PER; e++) atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(key_of(ee[e]), ident), bf)], 1u);
     }
   }
   for (; v < nvec; v += HIST_THREADS) {
     const uint4 w = __ldcs(vk + v);
-    const K* kk = reinterpret_cast<const K*>(&w);
+    const E* ee = reinterpret_cast<const E*>(&w);
 #pragma unroll
-    for (int e = 0; e < PER; e++) atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(kk[e], ident), bf)], 1u);
+    for (int e = 0; e < PER; e++) atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(key_of(ee[e]), ident), bf)], 1u);
   }
   __syncthreads();
   const uint32_t row0 = seg * P;
@@ -273,130 +377,83 @@ k_scan(uint32_t* __restrict__ hist, const uint32_t* __restrict__ rowsum, SegMap 
 
 // --------------------------------------------------------------------------
 // a8/a9: smem-staged, write-combined scatter (Fig. 4, P579-589).
-// Per tile of SC_TILE tuples: load (coalesced), compute the bucket, claim a
-// rank with a shared-memory atomic, exclusive-scan the tile's bucket counts,
-// reorder the tile in shared memory so each bucket is a consecutive run, then
-// write the runs with consecutive threads -> consecutive addresses (the runs
-// of one bucket continue where the previous tile's stopped, so L2 merges
-// partial sectors before they reach HBM).
-// --------------------------------------------------------------------------
-// The raw input tiles are streamed into shared memory by the bulk-copy
-// engine (cp.async.bulk, TMA 1-D) into a ring of SC_STAGES buffers tracked by
-// mbarriers, so HBM reads overlap the ranking / reordering / write-out of the
-// previous tile.  Tiles start at arbitrary element offsets: the copy covers
-// the enclosing 16-byte-aligned byte range and the tile is read at an offset.
-constexpr int SC_THREADS = 512;
-constexpr int SC_STAGES = 2;
-
-template <int KW, int PW> struct ScTile { static constexpr int T = (KW + PW) <= 8 ? 4096 : 2048; };
-
-__device__ __forceinline__ uint32_t smem_u32(const void* p) {
-  return static_cast<uint32_t>(__cvta_generic_to_shared(p));
-}
-__device__ __forceinline__ void mbar_init(uint64_t* bar, uint32_t count) {
-  asm volatile("mbarrier.init.shared::cta.b64 [%0], %1;" ::"r"(smem_u32(bar)), "r"(count));
-}
-__device__ __forceinline__ void mbar_expect_tx(uint64_t* bar, uint32_t bytes) {
-  asm volatile("mbarrier.arrive.expect_tx.shared::cta.b64 _, [%0], %1;" ::"r"(smem_u32(bar)), "r"(bytes)
-               : "memory");
-}
-__device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t phase) {
-  asm volatile(
-      "{\n .reg .pred p;\n WAIT_%=:\n"
-      " mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n"
-      " @!p bra WAIT_%=;\n}\n" ::"r"(smem_u32(bar)),
-      "r"(phase)
-      : "memory");
-}
-// producer-side wait: back off between polls so a warp that is far ahead
-// does not steal issue slots from the consumers
-__device__ __forceinline__ void mbar_wait_backoff(uint64_t* bar, uint32_t phase) {
-  uint32_t ok = 0;
-  while (true) {
-    asm volatile(
-        "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n selp.u32 %0, 1, 0, p;\n}\n"
-        : "=r"(ok)
-        : "r"(smem_u32(bar)), "r"(phase)
-        : "memory");
-    if (ok) return;
-    __nanosleep(256);
-  }
-}
-__device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t bytes, uint64_t* bar) {
-  asm volatile(
-      "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes [%0], [%1], %2, [%3];" ::"r"(
-          smem_u32(dst)),
-      "l"(src), "r"(bytes), "r"(smem_u32(bar))
-      : "memory");
-}
-
-__device__ __forceinline__ uint64_t policy_evict_first() {
-  uint64_t pol;
-  asm volatile("createpolicy.fractional.L2::evict_first.b64 %0, 1.0;" : "=l"(pol));
-  return pol;
-}
-__device__ __forceinline__ void bulk_g2s_ef(void* dst, const void* src, uint32_t bytes, uint64_t* bar,
-                                            uint64_t pol) {
-  asm volatile(
-      "cp.async.bulk.shared::cluster.global.mbarrier::complete_tx::bytes.L2::cache_hint [%0], [%1], %2, [%3], %4;" ::"r"(
-          smem_u32(dst)),
-      "l"(src), "r"(bytes), "r"(smem_u32(bar)), "l"(pol)
-      : "memory");
-}
-
-// one reordered tuple in shared memory (a single random-position store)
-template <int KW, int PW>
-struct alignas((KW + PW) <= 8 ? 8 : 16) ScPair {
-  typename UW<KW>::T k;
-  typename UW<PW>::T v;
-};
-
-template <int KW, int PW>
-__host__ __device__ constexpr size_t scatter_smem_bytes(uint32_t P) {
-  constexpr int T = ScTile<KW, PW>::T;
-  return (size_t)SC_STAGES * ((size_t)T * KW + 32 + (size_t)T * PW + 32)  // raw ring
-         + (size_t)T * sizeof(ScPair<KW, PW>)                              // reordered tile
-         + (size_t)P * 16 + 64 * 4 + SC_STAGES * 8 + 64;
-}
-
-// issue the bulk copies of tile [t0, t0+tn) into ring stage s (the enclosing
-// 16-byte-aligned byte ranges; the consumer reads at the residual offset)
-template <int KW, int PW>
-__device__ __forceinline__ void sc_issue(const void* ik, const void* ip, uint32_t t0, uint32_t tn,
-                                         unsigned char* rk, unsigned char* rp, uint64_t* bar, uint64_t pol) {
-  const uintptr_t ka = reinterpret_cast<uintptr_t>(ik) + (uintptr_t)t0 * KW;
-  const uintptr_t pa = reinterpret_cast<uintptr_t>(ip) + (uintptr_t)t0 * PW;
-  const uintptr_t k0 = ka & ~(uintptr_t)15, k1 = (ka + (uintptr_t)tn * KW + 15) & ~(uintptr_t)15;
-  const uintptr_t p0 = pa & ~(uintptr_t)15, p1 = (pa + (uintptr_t)tn * PW + 15) & ~(uintptr_t)15;
-  mbar_expect_tx(bar, (uint32_t)((k1 - k0) + (p1 - p0)));
-  bulk_g2s_ef(rk, reinterpret_cast<const void*>(k0), (uint32_t)(k1 - k0), bar, pol);
-  bulk_g2s_ef(rp, reinterpret_cast<const void*>(p0), (uint32_t)(p1 - p0), bar, pol);
-}
-
+// "we read a chunk of the input (at a time) in the scratchpad and reorganize
+// it in such a way that elements belonging to the same output partition are
+// located in consecutive scratchpad entries.  Then, we scan the scratchpad and
+// write each tuple to its corresponding output partition" (P579-584).
+//
+// Per tile of T tuples: the bulk-copy engine (cp.async.bulk + mbarrier, a
+// STAGES-deep ring) streams the raw tile into shared memory while the previous
+// tile is processed; phase 1 ranks each tuple inside its bucket with a
+// shared-memory atomic; phase 2 scans the tile's bucket counts and advances
+// the per-bucket HBM cursors; phase 3 places every tuple at its bucket run in
+// the reordered tile; phase 4 writes the runs with consecutive threads on
+// consecutive addresses.  The runs of a bucket continue where the previous
+// tile's stopped, so L2 merges partial sectors before they reach HBM.
+//
 // Odd chunks fill their per-bucket regions back to front: the sector shared
 // by the end of region (p, j) and the start of region (p, j+1) is then written
 // by both neighbours at the same moment of their lifetimes (both at the start,
 // or both at the end), so L2 merges it instead of evicting a half-written
 // sector and paying a DRAM read-modify-write.
-template <int KW, int PW>
-__global__ void __launch_bounds__(SC_THREADS, 2)
-k_scatter(const typename UW<KW>::T* __restrict__ ik, const typename UW<PW>::T* __restrict__ ip,
-          SegMap m, BitField bf, int ident, uint32_t P, const uint32_t* __restrict__ offsets,
-          typename UW<KW>::T* __restrict__ ok, typename UW<PW>::T* __restrict__ op) {
+// --------------------------------------------------------------------------
+template <int NT_, int ITEMS_, int STAGES_>
+struct ScCfg {
+  static constexpr int NT = NT_, ITEMS = ITEMS_, STAGES = STAGES_, T = NT_ * ITEMS_;
+};
+
+template <int KW, int PW, bool AOS, class C>
+struct ScLayout {
+  using Tp = Tup<KW, PW>;
+  static constexpr int T = C::T;
+  // raw landing buffer per stage: AoS tile, or key column + payload column
+  static constexpr size_t RK = AOS ? (size_t)T * sizeof(Tp) + 32 : (size_t)T * KW + 32;
+  static constexpr size_t RP = AOS ? 0 : (size_t)T * PW + 32;
+  static constexpr size_t RAW = (RK + RP + 15) / 16 * 16;
+  static __host__ __device__ constexpr size_t bytes(uint32_t P) {
+    return C::STAGES * RAW + (size_t)T * sizeof(Tp) + (size_t)((P + 3) & ~3u) * 16 + 64 * 4 + C::STAGES * 8 + 64;
+  }
+};
+
+template <int KW, int PW, bool AOS, class C>
+__device__ __forceinline__ void sc_issue(const PartIn& in, uint32_t t0, uint32_t tn, unsigned char* raw,
+                                         uint64_t* bar, uint64_t pol) {
+  using L = ScLayout<KW, PW, AOS, C>;
+  uint32_t tx = 0;
+  if constexpr (AOS) {
+    // expect_tx must precede the copies' completion: compute the size first
+    const uintptr_t a = reinterpret_cast<uintptr_t>(static_cast<const Tup<KW, PW>*>(in.t) + t0);
+    const uintptr_t a0 = a & ~(uintptr_t)15, a1 = (a + (size_t)tn * sizeof(Tup<KW, PW>) + 15) & ~(uintptr_t)15;
+    mbar_expect_tx(bar, (uint32_t)(a1 - a0));
+    bulk_g2s_any(raw, static_cast<const Tup<KW, PW>*>(in.t) + t0, (size_t)tn * sizeof(Tup<KW, PW>), bar, pol, &tx);
+  } else {
+    const uintptr_t ka = reinterpret_cast<uintptr_t>(static_cast<const char*>(in.k) + (size_t)t0 * KW);
+    const uintptr_t pa = reinterpret_cast<uintptr_t>(static_cast<const char*>(in.p) + (size_t)t0 * PW);
+    const uintptr_t k0 = ka & ~(uintptr_t)15, k1 = (ka + (size_t)tn * KW + 15) & ~(uintptr_t)15;
+    const uintptr_t p0 = pa & ~(uintptr_t)15, p1 = (pa + (size_t)tn * PW + 15) & ~(uintptr_t)15;
+    mbar_expect_tx(bar, (uint32_t)((k1 - k0) + (p1 - p0)));
+    bulk_g2s_any(raw, reinterpret_cast<const void*>(ka), (size_t)tn * KW, bar, pol, &tx);
+    bulk_g2s_any(raw + L::RK, reinterpret_cast<const void*>(pa), (size_t)tn * PW, bar, pol, &tx);
+  }
+}
+
+template <int KW, int PW, bool AOS, class C>
+__global__ void __launch_bounds__(C::NT, 1024 / C::NT)
+k_scatter(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, const uint32_t* __restrict__ offsets,
+          Tup<KW, PW>* __restrict__ out) {
   using K = typename UW<KW>::T;
   using V = typename UW<PW>::T;
-  using Pair = ScPair<KW, PW>;
-  constexpr int T = ScTile<KW, PW>::T;
-  constexpr int ITEMS = T / SC_THREADS;
-  constexpr int RK = T * KW + 32, RP = T * PW + 32;
+  using Tp = Tup<KW, PW>;
+  using L = ScLayout<KW, PW, AOS, C>;
+  constexpr int NT = C::NT, T = C::T, ITEMS = C::ITEMS, STAGES = C::STAGES;
   extern __shared__ __align__(128) unsigned char smem[];
-  unsigned char* raw = smem;                                            // [S][RK | RP]
-  Pair* s_pair = reinterpret_cast<Pair*>(smem + SC_STAGES * (RK + RP));
-  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_pair + T);
-  uint32_t* s_st = s_cnt + P;    // tile start of the bucket's run
-  uint32_t* s_cur = s_st + P;    // absolute write cursor (next free / one past next free if backward)
-  uint32_t* s_dlt = s_cur + P;   // HBM run start - tile run start
-  uint32_t* s_wt = s_dlt + P;    // warp totals [16]
+  unsigned char* raw = smem;                                            // [STAGES][RAW]
+  Tp* s_tile = reinterpret_cast<Tp*>(smem + STAGES * L::RAW);           // reordered tile
+  const uint32_t P4 = (P + 3) & ~3u;                  // keep the arrays below 16-byte aligned
+  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_tile + T);
+  uint2* s_sd = reinterpret_cast<uint2*>(s_cnt + P4);  // {tile start of run, HBM run start - tile start}
+  uint32_t* s_cur = reinterpret_cast<uint32_t*>(s_sd + P4);  // HBM write cursor per bucket
+  uint32_t* s_wt = s_cur + P4;                        // warp totals
   uint64_t* bar = reinterpret_cast<uint64_t*>(s_wt + 64);
 
   uint32_t seg, j, lo, hi;
@@ -405,49 +462,69 @@ k_scatter(const typename UW<KW>::T* __restrict__ ik, const typename UW<PW>::T* _
   const uint32_t row0 = seg * P;
   const size_t nflat = (size_t)m.nseg * P * m.cps;
   const uint32_t ntiles = (hi - lo + T - 1) / T;
-  for (uint32_t p = threadIdx.x; p < P; p += SC_THREADS) {
-    const size_t f = (size_t)(row0 + p) * m.cps + j;
-    s_cur[p] = backward ? (f + 1 < nflat ? offsets[f + 1] : m.n) : offsets[f];
-    s_cnt[p] = 0;
-  }
   uint64_t pol = 0;
   if (threadIdx.x == 0) {
     pol = policy_evict_first();
-    for (int s = 0; s < SC_STAGES; s++) mbar_init(&bar[s], 1);
+    for (int s = 0; s < STAGES; s++) mbar_init(&bar[s], 1);
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
-    for (uint32_t t = 0; t < (uint32_t)SC_STAGES && t < ntiles; t++) {
+    for (uint32_t t = 0; t < (uint32_t)STAGES && t < ntiles; t++) {
       const uint32_t t0 = lo + t * T;
-      sc_issue<KW, PW>(ik, ip, t0, min((uint32_t)T, hi - t0), raw + t * (RK + RP), raw + t * (RK + RP) + RK,
-                       &bar[t], pol);
+      sc_issue<KW, PW, AOS, C>(in, t0, min((uint32_t)T, hi - t0), raw + t * L::RAW, &bar[t], pol);
     }
+  }
+  for (uint32_t p = threadIdx.x; p < P; p += NT) {
+    const size_t f = (size_t)(row0 + p) * m.cps + j;
+    s_cur[p] = backward ? (f + 1 < nflat ? offsets[f + 1] : m.n) : offsets[f];
+    s_cnt[p] = 0;
   }
   __syncthreads();
 
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
   for (uint32_t t = 0; t < ntiles; t++) {
-    const uint32_t s = t % SC_STAGES, ph = (t / SC_STAGES) & 1;
+    const uint32_t s = t % STAGES, ph = (t / STAGES) & 1;
     const uint32_t t0 = lo + t * T, tn = min((uint32_t)T, hi - t0);
-    const unsigned char* rk = raw + s * (RK + RP);
-    const unsigned char* rp = rk + RK;
-    const K* tk = reinterpret_cast<const K*>(rk + ((reinterpret_cast<uintptr_t>(ik) + (uintptr_t)t0 * KW) & 15));
-    const V* tp = reinterpret_cast<const V*>(rp + ((reinterpret_cast<uintptr_t>(ip) + (uintptr_t)t0 * PW) & 15));
+    const unsigned char* rb = raw + s * L::RAW;
+    const K* tk;
+    const V* tp;
+    const Tp* tt;
+    if constexpr (AOS) {
+      tt = reinterpret_cast<const Tp*>(rb + (reinterpret_cast<uintptr_t>(static_cast<const Tp*>(in.t) + t0) & 15));
+    } else {
+      tk = reinterpret_cast<const K*>(rb + ((reinterpret_cast<uintptr_t>(in.k) + (uintptr_t)t0 * KW) & 15));
+      tp = reinterpret_cast<const V*>(rb + L::RK + ((reinterpret_cast<uintptr_t>(in.p) + (uintptr_t)t0 * PW) & 15));
+    }
+    auto load = [&](uint32_t i) -> Tp {
+      if constexpr (AOS) return tt[i];
+      else { Tp x; x.k = tk[i]; x.v = tp[i]; return x; }
+    };
     mbar_wait(&bar[s], ph);
-    // phase 1: bucket + rank (shared-memory atomic claim); keys stay in registers
+    // phase 1: bucket + rank (shared-memory atomic claim); tuples stay in registers
+    Tp x[ITEMS];
     uint32_t br[ITEMS];
-    K kr[ITEMS];
+    const bool full = tn == (uint32_t)T;
+    if (full) {
 #pragma unroll
-    for (int u = 0; u < ITEMS; u++) {
-      const uint32_t i = u * SC_THREADS + threadIdx.x;
-      if (i < tn) {
-        kr[u] = tk[i];
-        const uint32_t b = bucket_of(part_hash<KW>(kr[u], ident), bf);
+      for (int u = 0; u < ITEMS; u++) x[u] = load(u * NT + threadIdx.x);
+#pragma unroll
+      for (int u = 0; u < ITEMS; u++) {
+        const uint32_t b = bucket_of(part_hash<KW>(x[u].k, ident), bf);
         br[u] = (b << 16) | atomicAdd(&s_cnt[b], 1u);
       }
+    } else {
+#pragma unroll
+      for (int u = 0; u < ITEMS; u++) {
+        const uint32_t i = u * NT + threadIdx.x;
+        if (i < tn) {
+          x[u] = load(i);
+          const uint32_t b = bucket_of(part_hash<KW>(x[u].k, ident), bf);
+          br[u] = (b << 16) | atomicAdd(&s_cnt[b], 1u);
+        }
+      }
     }
-    __syncthreads();  // A
+    __syncthreads();  // A: counts complete
     // phase 2: exclusive scan of the tile's bucket counts; advance the cursors
     {
-      const uint32_t per = (P + SC_THREADS - 1) / SC_THREADS;
+      const uint32_t per = (P + NT - 1) / NT;
       const uint32_t b0 = min(threadIdx.x * per, P), b1 = min(b0 + per, P);
       uint32_t sum = 0;
       for (uint32_t b = b0; b < b1; b++) sum += s_cnt[b];
@@ -459,41 +536,42 @@ k_scatter(const typename UW<KW>::T* __restrict__ ik, const typename UW<PW>::T* _
       for (uint32_t b = b0; b < b1; b++) {
         const uint32_t c = s_cnt[b], cur = s_cur[b];
         const uint32_t run = backward ? cur - c : cur;
-        s_st[b] = ex;
-        s_dlt[b] = run - ex;
+        s_sd[b] = make_uint2(ex, run - ex);
         s_cur[b] = backward ? cur - c : cur + c;
         s_cnt[b] = 0;
         ex += c;
       }
     }
-    __syncthreads();  // B
+    __syncthreads();  // B: run starts known
     // phase 3: reorder the tile in shared memory, bucket runs consecutive
+    if (full) {
 #pragma unroll
-    for (int u = 0; u < ITEMS; u++) {
-      const uint32_t i = u * SC_THREADS + threadIdx.x;
-      if (i < tn) {
-        const uint32_t pos = s_st[br[u] >> 16] + (br[u] & 0xFFFFu);
-        Pair pr;
-        pr.k = kr[u];
-        pr.v = tp[i];
-        s_pair[pos] = pr;
-      }
+      for (int u = 0; u < ITEMS; u++) s_tile[s_sd[br[u] >> 16].x + (br[u] & 0xFFFFu)] = x[u];
+    } else {
+#pragma unroll
+      for (int u = 0; u < ITEMS; u++)
+        if (u * NT + threadIdx.x < tn) s_tile[s_sd[br[u] >> 16].x + (br[u] & 0xFFFFu)] = x[u];
     }
     __syncthreads();  // C: raw stage s is free, the reordered tile is complete
-    if (threadIdx.x == 0 && t + SC_STAGES < ntiles) {
-      const uint32_t n0 = lo + (t + SC_STAGES) * T;
-      sc_issue<KW, PW>(ik, ip, n0, min((uint32_t)T, hi - n0), raw + s * (RK + RP), raw + s * (RK + RP) + RK,
-                       &bar[s], pol);
+    if (threadIdx.x == 0 && t + STAGES < ntiles) {
+      const uint32_t n0 = lo + (t + STAGES) * T;
+      sc_issue<KW, PW, AOS, C>(in, n0, min((uint32_t)T, hi - n0), raw + s * L::RAW, &bar[s], pol);
     }
     // phase 4: write the runs; consecutive threads -> consecutive addresses
     // (the bucket is recomputed from the key: ALU is cheaper than another
     // random shared-memory store + load)
-#pragma unroll 4
-    for (uint32_t i = threadIdx.x; i < tn; i += SC_THREADS) {
-      const Pair pr = s_pair[i];
-      const uint32_t dst = s_dlt[bucket_of(part_hash<KW>(pr.k, ident), bf)] + i;
-      ok[dst] = pr.k;
-      op[dst] = pr.v;
+    if (full) {
+#pragma unroll
+      for (int u = 0; u < ITEMS; u++) {
+        const uint32_t i = u * NT + threadIdx.x;
+        const Tp y = s_tile[i];
+        out[s_sd[bucket_of(part_hash<KW>(y.k, ident), bf)].y + i] = y;
+      }
+    } else {
+      for (uint32_t i = threadIdx.x; i < tn; i += NT) {
+        const Tp y = s_tile[i];
+        out[s_sd[bucket_of(part_hash<KW>(y.k, ident), bf)].y + i] = y;
+      }
     }
   }
 }
@@ -534,12 +612,6 @@ k_worklist(const uint32_t* __restrict__ bR, const uint32_t* __restrict__ bS, uin
 // optional materialisation through a block-aggregated output claim
 // ("Buffer output ... ATOMICS!", Fig. 3 P488-493).
 //
-// Persistent CTAs pull items from an atomic counter.  Shared memory holds the
-// R chunk (keys, payloads), next[] chain links (u16) and epoch-tagged chain
-// heads[2^slot_bits] (u32: epoch<<16 | index), so no head reset is needed
-// between builds.  The slot uses hash bits above the radix bits (every tuple
-// of a co-partition shares those).
-// --------------------------------------------------------------------------
 // Warp-specialised pipeline (the Blackwell producer/consumer idiom):
 //   * a producer warp walks this CTA's static share of the work list
 //     (items blockIdx.x, +gridDim.x, ...; co-partitions are near-uniform, so a
@@ -547,16 +619,17 @@ k_worklist(const uint32_t* __restrict__ bR, const uint32_t* __restrict__ bS, uin
 //     into a 2-deep ring of shared-memory buffers with the bulk-copy engine
 //     (cp.async.bulk + mbarrier), one "stage" per (R chunk, S slice);
 //   * 8 consumer warps build a chained table over the landed chunk (heads
-//     reset per stage, atomicExch on the heads, u16 next links) and probe the S
-//     slice, streaming S from HBM with 4 independent loads per thread.
+//     reset per stage, atomicExch on the heads, u16 next links) and probe the
+//     S slice, streaming S tuples from HBM, 4 independent loads per thread.
 // The next stage's R chunk lands while the current one is probed.
 //
 // The slot of a key inside the smem table is a multiplicative hash of the key
 // (2 instructions) rather than more bits of the partition hash: every tuple of
 // a co-partition shares the partition bits, and any function of the key that
-// spreads them works -- the result does not depend on it.
-// For each S tuple the chain is walked to its end (bag semantics); the
-// aggregation body of a match runs with the lanes converged, once per round.
+// spreads them works -- the result does not depend on it.  For each S tuple
+// the chain is walked to its end (bag semantics); the aggregation body of a
+// match runs with the lanes converged, once per round.
+// --------------------------------------------------------------------------
 constexpr int JN_CONSUMERS = 256;
 constexpr int JN_THREADS = JN_CONSUMERS + 32;
 constexpr int JN_U = 4;
@@ -564,34 +637,30 @@ constexpr uint32_t JN_MAXCAP = 16384;
 constexpr uint32_t JN_NIL = 0xFFFFu;
 constexpr uint32_t JN_STOP = 0xFFFFFFFFu;
 
-template <int KW, int PRW, int PSW>
+template <int KW, int PRW>
 __host__ __device__ constexpr size_t join_smem_bytes(uint32_t cap, uint32_t slot_bits) {
-  return 2 * (((size_t)cap * KW + 32 + 15) / 16 * 16 + ((size_t)cap * PRW + 32 + 15) / 16 * 16)  // R ring
-         + ((size_t)cap * 2 + 15) / 16 * 16                                                        // next[]
-         + ((size_t)4 << slot_bits);                                                               // heads[]
+  return 2 * (((size_t)cap * sizeof(Tup<KW, PRW>) + 32 + 15) / 16 * 16)  // R ring
+         + ((size_t)cap * 2 + 15) / 16 * 16                                // next[]
+         + ((size_t)4 << slot_bits);                                       // heads[]
 }
 
 struct JoinArgs {
-  const void* rk; const void* rp; const void* sk; const void* sp;
+  const void* rt; const void* st;            // R / S tuples (AoS workspace)
   const uint32_t* bR; const uint32_t* bS;
-  const uint2* items; const uint32_t* n_items; uint32_t* item_ctr;
-  uint32_t cap; uint32_t slice; uint32_t slot_shift; uint32_t slot_bits; int ident;
-  unsigned long long* acc;       // [4] count, sum_r, sum_s, checksum
+  const uint2* items; const uint32_t* n_items;
+  uint32_t cap; uint32_t slice; uint32_t slot_bits;
+  unsigned long long* acc;                   // [4] count, sum_r, sum_s, checksum
   void* out_r; void* out_s; unsigned long long out_cap; unsigned long long* out_ctr;
 };
 
 struct JnStage {
   uint32_t nr;      // R tuples in the chunk (JN_STOP = no more stages)
-  uint32_t koff;    // byte offset of element 0 inside the key buffer
-  uint32_t poff;    // byte offset of element 0 inside the payload buffer
+  uint32_t off;     // byte offset of tuple 0 inside the ring buffer
   uint32_t s_lo, s_hi;
 };
 
 __device__ __forceinline__ void consumer_sync() {
   asm volatile("bar.sync 1, %0;" ::"n"(JN_CONSUMERS) : "memory");
-}
-__device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
-  asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
 }
 
 // slot of a key in the smem table: top slot_bits bits of key * odd constant
@@ -605,10 +674,9 @@ struct JnAcc {
   unsigned long long cnt = 0, sr = 0, ss = 0, sx = 0;
 };
 
-template <int KW, int PRW, int PSW>
+template <int KW, int PRW>
 struct JnTable {
-  const typename UW<KW>::T* k;     // R chunk keys (landing buffer)
-  const typename UW<PRW>::S* p;    // R chunk payloads
+  const Tup<KW, PRW>* r;    // R chunk (ring buffer)
   const uint16_t* next;
   const uint32_t* head;
   uint32_t sbits;
@@ -616,26 +684,25 @@ struct JnTable {
 
 // Probe U S tuples per consumer thread: j = base + u*256 + tid.
 template <int KW, int PRW, int PSW, bool MAT, int U>
-__device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, PSW>& t, const JoinArgs& a, uint32_t base,
+__device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const JoinArgs& a, uint32_t base,
                                                uint32_t s_hi, JnAcc& acc, uint32_t* s_wsum,
                                                unsigned long long* s_wbase) {
-  using K = typename UW<KW>::T;
+  using TS = Tup<KW, PSW>;
+  using PR = typename UW<PRW>::S;
   using PS = typename UW<PSW>::S;
-  const K* __restrict__ sk = static_cast<const K*>(a.sk);
-  const PS* __restrict__ sp = static_cast<const PS*>(a.sp);
+  const TS* __restrict__ sT = static_cast<const TS*>(a.st);
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-  K k[U];
-  PS v[U];
+  TS x[U];
   uint32_t e0[U];
 #pragma unroll
   for (int u = 0; u < U; u++) {
     const uint32_t j = base + u * JN_CONSUMERS + threadIdx.x;
-    if (j < s_hi) { k[u] = __ldcs(sk + j); v[u] = __ldcs(sp + j); }
+    if (j < s_hi) x[u] = ldcs_tup(sT + j);
   }
 #pragma unroll
   for (int u = 0; u < U; u++) {
     const uint32_t j = base + u * JN_CONSUMERS + threadIdx.x;
-    e0[u] = j < s_hi ? t.head[jn_slot<KW>(k[u], t.sbits)] : JN_NIL;
+    e0[u] = j < s_hi ? t.head[jn_slot<KW>(x[u].k, t.sbits)] : JN_NIL;
   }
   uint32_t c[U];
 #pragma unroll
@@ -645,11 +712,11 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, PSW>& t, c
     c[u] = 0;
     uint32_t e = e0[u];
     while (true) {
-      while (e != JN_NIL && t.k[e] != k[u]) e = t.next[e];
+      while (e != JN_NIL && t.r[e].k != x[u].k) e = t.next[e];
       const bool hit = e != JN_NIL;
       if (!__any_sync(0xffffffffu, hit)) break;
       if (hit) {
-        const int64_t pr = (int64_t)t.p[e], ps = (int64_t)v[u];
+        const int64_t pr = (int64_t)(PR)t.r[e].v, ps = (int64_t)(PS)x[u].v;
         c[u]++;
         acc.sr += (unsigned long long)pr;
         acc.ss += (unsigned long long)ps;
@@ -679,16 +746,15 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, PSW>& t, c
     }
     consumer_sync();
     const unsigned long long wb = s_wbase[warp];
-    using PR = typename UW<PRW>::S;
 #pragma unroll
     for (int u = 0; u < U; u++) {
       if (!c[u]) continue;
       unsigned long long pos = wb + before[u] + incl[u] - c[u];
       for (uint32_t e = e0[u]; e != JN_NIL; e = t.next[e]) {
-        if (t.k[e] == k[u]) {
+        if (t.r[e].k == x[u].k) {
           if (pos < a.out_cap) {
-            static_cast<PR*>(a.out_r)[pos] = t.p[e];
-            static_cast<PS*>(a.out_s)[pos] = v[u];
+            static_cast<PR*>(a.out_r)[pos] = (PR)t.r[e].v;
+            static_cast<PS*>(a.out_s)[pos] = (PS)x[u].v;
           }
           pos++;
         }
@@ -700,13 +766,12 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, PSW>& t, c
 template <int KW, int PRW, int PSW, bool MAT>
 __global__ void __launch_bounds__(JN_THREADS)
 k_build_probe(JoinArgs a) {
-  using K = typename UW<KW>::T;
-  using PR = typename UW<PRW>::S;
+  using TR = Tup<KW, PRW>;
   extern __shared__ __align__(128) unsigned char smem[];
-  const uint32_t RKB = (a.cap * KW + 32 + 15) / 16 * 16, RPB = (a.cap * PRW + 32 + 15) / 16 * 16;
-  unsigned char* ring = smem;                                           // [2][RKB | RPB]
-  uint16_t* s_next = reinterpret_cast<uint16_t*>(smem + 2 * (RKB + RPB));
-  uint32_t* s_head = reinterpret_cast<uint32_t*>(smem + 2 * (RKB + RPB) + ((size_t)a.cap * 2 + 15) / 16 * 16);
+  const uint32_t RB = ((uint32_t)(a.cap * sizeof(TR)) + 32 + 15) / 16 * 16;
+  unsigned char* ring = smem;                                           // [2][RB]
+  uint16_t* s_next = reinterpret_cast<uint16_t*>(smem + 2 * RB);
+  uint32_t* s_head = reinterpret_cast<uint32_t*>(smem + 2 * RB + ((size_t)a.cap * 2 + 15) / 16 * 16);
   __shared__ JnStage s_meta[2];
   __shared__ __align__(8) uint64_t full[2], empty[2];
   __shared__ uint32_t s_wsum[JN_CONSUMERS / 32];
@@ -728,8 +793,7 @@ k_build_probe(JoinArgs a) {
     if (lane == 0) {
       const uint64_t pol = policy_evict_first();
       const uint32_t n_items = *a.n_items;
-      const char* rkb = static_cast<const char*>(a.rk);
-      const char* rpb = static_cast<const char*>(a.rp);
+      const TR* rT = static_cast<const TR*>(a.rt);
       uint32_t stage = 0;
       for (uint32_t it = blockIdx.x; it < n_items; it += gridDim.x) {
         const uint2 item = a.items[it];
@@ -741,15 +805,11 @@ k_build_probe(JoinArgs a) {
           const uint32_t bi = stage & 1, ph = (stage >> 1) & 1;
           mbar_wait_backoff(&empty[bi], ph ^ 1);
           const uint32_t nr = min(a.cap, r_hi - c_lo);
-          const uintptr_t ka = reinterpret_cast<uintptr_t>(rkb + (size_t)c_lo * KW);
-          const uintptr_t pa = reinterpret_cast<uintptr_t>(rpb + (size_t)c_lo * PRW);
-          const uintptr_t k0 = ka & ~(uintptr_t)15, k1 = (ka + (size_t)nr * KW + 15) & ~(uintptr_t)15;
-          const uintptr_t p0 = pa & ~(uintptr_t)15, p1 = (pa + (size_t)nr * PRW + 15) & ~(uintptr_t)15;
-          s_meta[bi] = JnStage{nr, (uint32_t)(ka - k0), (uint32_t)(pa - p0), s_lo, s_hi};
-          unsigned char* kbuf = ring + bi * (RKB + RPB);
-          mbar_expect_tx(&full[bi], (uint32_t)((k1 - k0) + (p1 - p0)));
-          bulk_g2s_ef(kbuf, reinterpret_cast<const void*>(k0), (uint32_t)(k1 - k0), &full[bi], pol);
-          bulk_g2s_ef(kbuf + RKB, reinterpret_cast<const void*>(p0), (uint32_t)(p1 - p0), &full[bi], pol);
+          const uintptr_t ra = reinterpret_cast<uintptr_t>(rT + c_lo);
+          const uintptr_t r0 = ra & ~(uintptr_t)15, r1 = (ra + (size_t)nr * sizeof(TR) + 15) & ~(uintptr_t)15;
+          s_meta[bi] = JnStage{nr, (uint32_t)(ra - r0), s_lo, s_hi};
+          mbar_expect_tx(&full[bi], (uint32_t)(r1 - r0));
+          bulk_g2s(ring + bi * RB, reinterpret_cast<const void*>(r0), (uint32_t)(r1 - r0), &full[bi], pol);
         }
       }
       const uint32_t bi = stage & 1, ph = (stage >> 1) & 1;
@@ -768,16 +828,14 @@ k_build_probe(JoinArgs a) {
       mbar_wait(&full[bi], ph);
       const JnStage st = s_meta[bi];
       if (st.nr == JN_STOP) break;
-      const unsigned char* kbuf = ring + bi * (RKB + RPB);
-      const K* s_rk = reinterpret_cast<const K*>(kbuf + st.koff);
-      const PR* s_rp = reinterpret_cast<const PR*>(kbuf + RKB + st.poff);
+      const TR* r = reinterpret_cast<const TR*>(ring + bi * RB + st.off);
       consumer_sync();
       // ---- build (a11): chained table via atomicExch on the heads
       for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
-        s_next[i] = (uint16_t)atomicExch(&s_head[jn_slot<KW>(s_rk[i], a.slot_bits)], i);
+        s_next[i] = (uint16_t)atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], i);
       consumer_sync();
       // ---- probe (a12): stream the S slice
-      const JnTable<KW, PRW, PSW> tab{s_rk, s_rp, s_next, s_head, a.slot_bits};
+      const JnTable<KW, PRW> tab{r, s_next, s_head, a.slot_bits};
       uint32_t base = st.s_lo;
       for (; base + JN_U * JN_CONSUMERS <= st.s_hi; base += JN_U * JN_CONSUMERS)
         jn_probe_batch<KW, PRW, PSW, MAT, JN_U>(tab, a, base, st.s_hi, acc, s_wsum, s_wbase);
@@ -807,6 +865,17 @@ k_build_probe(JoinArgs a) {
     unsigned long long t = 0;
     for (int w = 0; w < JN_THREADS / 32; w++) t += s_red[threadIdx.x][w];
     if (t) atomicAdd(&a.acc[threadIdx.x], t);
+  }
+}
+
+// unpack AoS tuples into key / payload columns (debug entry point only)
+template <int KW, int PW>
+__global__ void k_unpack(const Tup<KW, PW>* __restrict__ t, uint32_t n, typename UW<KW>::T* __restrict__ k,
+                         typename UW<PW>::T* __restrict__ p) {
+  for (uint32_t i = blockIdx.x * blockDim.x + threadIdx.x; i < n; i += gridDim.x * blockDim.x) {
+    const Tup<KW, PW> x = t[i];
+    k[i] = x.k;
+    p[i] = x.v;
   }
 }
 
