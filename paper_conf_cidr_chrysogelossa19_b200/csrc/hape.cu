@@ -289,16 +289,19 @@ static hape_status scatter_v(hape_join* h, const Src& s, SegMap m, BitField bf, 
   static int v = [] { const char* e = getenv("HAPE_SC"); return e ? atoi(e) : -1; }();
   if constexpr (KW + PW <= 8) {
     switch (v) {
-      case 1: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 1>>(h, s, m, bf, P, offs, out);
-      case 2: return scatter_t<KW, PW, AOS, ScCfg<256, 16, 2>>(h, s, m, bf, P, offs, out);
-      case 3: return scatter_t<KW, PW, AOS, ScCfg<1024, 8, 1>>(h, s, m, bf, P, offs, out);
-      case 4: return scatter_t<KW, PW, AOS, ScCfg<256, 8, 2>>(h, s, m, bf, P, offs, out);
-      default: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 2>>(h, s, m, bf, P, offs, out);
+      case 1: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2>>(h, s, m, bf, P, offs, out);
+      case 2: return scatter_t<KW, PW, AOS, ScCfg<256, 16, 2, 3>>(h, s, m, bf, P, offs, out);
+      case 3: return scatter_t<KW, PW, AOS, ScCfg<256, 16, 3, 2>>(h, s, m, bf, P, offs, out);
+      case 4: return scatter_t<KW, PW, AOS, ScCfg<512, 16, 2, 1>>(h, s, m, bf, P, offs, out);
+      case 5: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 2, 2, true>>(h, s, m, bf, P, offs, out);
+      case 6: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2, true>>(h, s, m, bf, P, offs, out);
+      case 7: return scatter_t<KW, PW, AOS, ScCfg<256, 16, 2, 2, true>>(h, s, m, bf, P, offs, out);
+      default: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 2, 3>>(h, s, m, bf, P, offs, out);
     }
   } else {
     switch (v) {
-      case 1: return scatter_t<KW, PW, AOS, ScCfg<512, 4, 2>>(h, s, m, bf, P, offs, out);
-      default: return scatter_t<KW, PW, AOS, ScCfg<256, 8, 2>>(h, s, m, bf, P, offs, out);
+      case 1: return scatter_t<KW, PW, AOS, ScCfg<256, 8, 3, 2>>(h, s, m, bf, P, offs, out);
+      default: return scatter_t<KW, PW, AOS, ScCfg<256, 8, 2, 3>>(h, s, m, bf, P, offs, out);
     }
   }
 }

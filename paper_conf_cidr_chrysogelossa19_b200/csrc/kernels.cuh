@@ -222,18 +222,18 @@ __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t phase) {
       "r"(phase)
       : "memory");
 }
-// producer-side wait: back off between polls so a warp that is far ahead
-// does not steal issue slots from the consumers
+// producer-side wait: the thread is suspended inside try_wait (time-limit
+// hint) instead of polling, so a warp that is far ahead does not steal issue
+// slots from the consumers
 __device__ __forceinline__ void mbar_wait_backoff(uint64_t* bar, uint32_t phase) {
   uint32_t ok = 0;
   while (true) {
     asm volatile(
-        "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2;\n selp.u32 %0, 1, 0, p;\n}\n"
+        "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2, %3;\n selp.u32 %0, 1, 0, p;\n}\n"
         : "=r"(ok)
-        : "r"(smem_u32(bar)), "r"(phase)
+        : "r"(smem_u32(bar)), "r"(phase), "r"(1000000u)
         : "memory");
     if (ok) return;
-    __nanosleep(256);
   }
 }
 __device__ __forceinline__ uint64_t policy_evict_first() {
@@ -397,21 +397,26 @@ k_scan(uint32_t* __restrict__ hist, const uint32_t* __restrict__ rowsum, SegMap 
 // or both at the end), so L2 merges it instead of evicting a half-written
 // sector and paying a DRAM read-modify-write.
 // --------------------------------------------------------------------------
-template <int NT_, int ITEMS_, int STAGES_>
+template <int NT_, int ITEMS_, int STAGES_, int MINB_ = 1024 / NT_, bool DST_ = false>
 struct ScCfg {
-  static constexpr int NT = NT_, ITEMS = ITEMS_, STAGES = STAGES_, T = NT_ * ITEMS_;
+  static constexpr int NT = NT_, ITEMS = ITEMS_, STAGES = STAGES_, T = NT_ * ITEMS_, MINB = MINB_;
+  static constexpr bool DST = DST_;  // reorder phase stores each tuple's HBM slot
 };
 
 template <int KW, int PW, bool AOS, class C>
 struct ScLayout {
   using Tp = Tup<KW, PW>;
   static constexpr int T = C::T;
-  // raw landing buffer per stage: AoS tile, or key column + payload column
+  // landing buffer per stage: AoS tile, or key column + payload column.  The
+  // reordered tile is written back into the same buffer (in place: every
+  // tuple is in registers once ranked), so a stage costs T tuples of smem.
   static constexpr size_t RK = AOS ? (size_t)T * sizeof(Tp) + 32 : (size_t)T * KW + 32;
   static constexpr size_t RP = AOS ? 0 : (size_t)T * PW + 32;
-  static constexpr size_t RAW = (RK + RP + 15) / 16 * 16;
+  static constexpr size_t RAW0 = (RK + RP + 15) / 16 * 16;
+  static constexpr size_t RAW = RAW0 > (size_t)T * sizeof(Tp) ? RAW0 : (size_t)T * sizeof(Tp);
   static __host__ __device__ constexpr size_t bytes(uint32_t P) {
-    return C::STAGES * RAW + (size_t)T * sizeof(Tp) + (size_t)((P + 3) & ~3u) * 16 + 64 * 4 + C::STAGES * 8 + 64;
+    return C::STAGES * RAW + (C::DST ? (size_t)T * 4 : 0) + (size_t)((P + 3) & ~3u) * 16 + 64 * 4 +
+           C::STAGES * 8 + 64;
   }
 };
 
@@ -438,7 +443,7 @@ __device__ __forceinline__ void sc_issue(const PartIn& in, uint32_t t0, uint32_t
 }
 
 template <int KW, int PW, bool AOS, class C>
-__global__ void __launch_bounds__(C::NT, 1024 / C::NT)
+__global__ void __launch_bounds__(C::NT, C::MINB)
 k_scatter(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, const uint32_t* __restrict__ offsets,
           Tup<KW, PW>* __restrict__ out) {
   using K = typename UW<KW>::T;
@@ -448,11 +453,12 @@ k_scatter(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, const uint32_
   constexpr int NT = C::NT, T = C::T, ITEMS = C::ITEMS, STAGES = C::STAGES;
   extern __shared__ __align__(128) unsigned char smem[];
   unsigned char* raw = smem;                                            // [STAGES][RAW]
-  Tp* s_tile = reinterpret_cast<Tp*>(smem + STAGES * L::RAW);           // reordered tile
   const uint32_t P4 = (P + 3) & ~3u;                  // keep the arrays below 16-byte aligned
-  uint32_t* s_cnt = reinterpret_cast<uint32_t*>(s_tile + T);
-  uint2* s_sd = reinterpret_cast<uint2*>(s_cnt + P4);  // {tile start of run, HBM run start - tile start}
-  uint32_t* s_cur = reinterpret_cast<uint32_t*>(s_sd + P4);  // HBM write cursor per bucket
+  uint32_t* s_dst = reinterpret_cast<uint32_t*>(smem + STAGES * L::RAW);  // DST only
+  uint32_t* s_cnt = s_dst + (C::DST ? T : 0);
+  uint32_t* s_st = s_cnt + P4;                        // tile start of the bucket's run
+  uint32_t* s_dl = s_st + P4;                         // HBM run start - tile start
+  uint32_t* s_cur = s_dl + P4;                        // HBM write cursor per bucket
   uint32_t* s_wt = s_cur + P4;                        // warp totals
   uint64_t* bar = reinterpret_cast<uint64_t*>(s_wt + 64);
 
@@ -483,7 +489,8 @@ k_scatter(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, const uint32_
   for (uint32_t t = 0; t < ntiles; t++) {
     const uint32_t s = t % STAGES, ph = (t / STAGES) & 1;
     const uint32_t t0 = lo + t * T, tn = min((uint32_t)T, hi - t0);
-    const unsigned char* rb = raw + s * L::RAW;
+    unsigned char* rb = raw + s * L::RAW;
+    Tp* s_tile = reinterpret_cast<Tp*>(rb);            // reordered tile (in place)
     const K* tk;
     const V* tp;
     const Tp* tt;
@@ -498,7 +505,7 @@ k_scatter(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, const uint32_
       else { Tp x; x.k = tk[i]; x.v = tp[i]; return x; }
     };
     mbar_wait(&bar[s], ph);
-    // phase 1: bucket + rank (shared-memory atomic claim); tuples stay in registers
+    // phase 1: bucket + rank (shared-memory atomic claim); tuples -> registers
     Tp x[ITEMS];
     uint32_t br[ITEMS];
     const bool full = tn == (uint32_t)T;
@@ -521,7 +528,13 @@ k_scatter(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, const uint32_
         }
       }
     }
-    __syncthreads();  // A: counts complete
+    __syncthreads();  // A: counts complete; the whole tile is in registers
+    // the previous tile's buffer is now free (its write-out finished before A)
+    if (threadIdx.x == 0 && t >= 1 && t - 1 + STAGES < ntiles) {
+      const uint32_t n0 = lo + (t - 1 + STAGES) * T;
+      sc_issue<KW, PW, AOS, C>(in, n0, min((uint32_t)T, hi - n0), raw + ((t - 1) % STAGES) * L::RAW,
+                               &bar[(t - 1) % STAGES], pol);
+    }
     // phase 2: exclusive scan of the tile's bucket counts; advance the cursors
     {
       const uint32_t per = (P + NT - 1) / NT;
@@ -536,41 +549,52 @@ k_scatter(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, const uint32_
       for (uint32_t b = b0; b < b1; b++) {
         const uint32_t c = s_cnt[b], cur = s_cur[b];
         const uint32_t run = backward ? cur - c : cur;
-        s_sd[b] = make_uint2(ex, run - ex);
+        s_st[b] = ex;
+        s_dl[b] = run - ex;
         s_cur[b] = backward ? cur - c : cur + c;
         s_cnt[b] = 0;
         ex += c;
       }
     }
     __syncthreads();  // B: run starts known
-    // phase 3: reorder the tile in shared memory, bucket runs consecutive
+    // phase 3: reorder the tile in shared memory (in place), bucket runs consecutive
     if (full) {
 #pragma unroll
-      for (int u = 0; u < ITEMS; u++) s_tile[s_sd[br[u] >> 16].x + (br[u] & 0xFFFFu)] = x[u];
+      for (int u = 0; u < ITEMS; u++) {
+        const uint32_t pos = s_st[br[u] >> 16] + (br[u] & 0xFFFFu);
+        s_tile[pos] = x[u];
+        if constexpr (C::DST) s_dst[pos] = s_dl[br[u] >> 16] + pos;
+      }
     } else {
 #pragma unroll
       for (int u = 0; u < ITEMS; u++)
-        if (u * NT + threadIdx.x < tn) s_tile[s_sd[br[u] >> 16].x + (br[u] & 0xFFFFu)] = x[u];
+        if (u * NT + threadIdx.x < tn) {
+          const uint32_t pos = s_st[br[u] >> 16] + (br[u] & 0xFFFFu);
+          s_tile[pos] = x[u];
+          if constexpr (C::DST) s_dst[pos] = s_dl[br[u] >> 16] + pos;
+        }
     }
-    __syncthreads();  // C: raw stage s is free, the reordered tile is complete
-    if (threadIdx.x == 0 && t + STAGES < ntiles) {
-      const uint32_t n0 = lo + (t + STAGES) * T;
-      sc_issue<KW, PW, AOS, C>(in, n0, min((uint32_t)T, hi - n0), raw + s * L::RAW, &bar[s], pol);
-    }
+    // generic-proxy writes to a buffer the bulk-copy engine refills later
+    asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+    __syncthreads();  // C: the reordered tile is complete
     // phase 4: write the runs; consecutive threads -> consecutive addresses
     // (the bucket is recomputed from the key: ALU is cheaper than another
     // random shared-memory store + load)
+    auto dst_of = [&](uint32_t i, const Tp& y) -> uint32_t {
+      if constexpr (C::DST) return s_dst[i];
+      else return s_dl[bucket_of(part_hash<KW>(y.k, ident), bf)] + i;
+    };
     if (full) {
 #pragma unroll
       for (int u = 0; u < ITEMS; u++) {
         const uint32_t i = u * NT + threadIdx.x;
         const Tp y = s_tile[i];
-        out[s_sd[bucket_of(part_hash<KW>(y.k, ident), bf)].y + i] = y;
+        out[dst_of(i, y)] = y;
       }
     } else {
       for (uint32_t i = threadIdx.x; i < tn; i += NT) {
         const Tp y = s_tile[i];
-        out[s_sd[bucket_of(part_hash<KW>(y.k, ident), bf)].y + i] = y;
+        out[dst_of(i, y)] = y;
       }
     }
   }
@@ -680,6 +704,7 @@ struct JnTable {
   const uint16_t* next;
   const uint32_t* head;
   uint32_t sbits;
+  bool dup;                 // the chunk holds some key twice (bag semantics path)
 };
 
 // Probe U S tuples per consumer thread: j = base + u*256 + tid.
@@ -704,28 +729,58 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
     const uint32_t j = base + u * JN_CONSUMERS + threadIdx.x;
     e0[u] = j < s_hi ? t.head[jn_slot<KW>(x[u].k, t.sbits)] : JN_NIL;
   }
+  // 1) find each tuple's first match: the U chain walks advance together, so
+  //    their dependent shared loads overlap (no warp-wide synchronisation)
+  uint32_t e[U];
+  bool act[U];
+#pragma unroll
+  for (int u = 0; u < U; u++) {
+    e[u] = e0[u];
+    act[u] = e[u] != JN_NIL && t.r[e[u]].k != x[u].k;
+  }
+  while (true) {
+    bool any = false;
+#pragma unroll
+    for (int u = 0; u < U; u++) any |= act[u];
+    if (!any) break;
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      if (act[u]) {
+        e[u] = t.next[e[u]];
+        act[u] = e[u] != JN_NIL && t.r[e[u]].k != x[u].k;
+      }
+    }
+  }
+  // 2) aggregate the first matches: U independent predicated bodies (the
+  //    64-bit mixing chains interleave)
   uint32_t c[U];
 #pragma unroll
   for (int u = 0; u < U; u++) {
-    // walk to the next match (divergent, cheap), then run the aggregation
-    // body once per round with every lane that found one (converged)
-    c[u] = 0;
-    uint32_t e = e0[u];
-    while (true) {
-      while (e != JN_NIL && t.r[e].k != x[u].k) e = t.next[e];
-      const bool hit = e != JN_NIL;
-      if (!__any_sync(0xffffffffu, hit)) break;
-      if (hit) {
-        const int64_t pr = (int64_t)(PR)t.r[e].v, ps = (int64_t)(PS)x[u].v;
-        c[u]++;
-        acc.sr += (unsigned long long)pr;
-        acc.ss += (unsigned long long)ps;
-        acc.sx += pair_mix(pr, ps);
-        e = t.next[e];
+    c[u] = e[u] != JN_NIL;
+    if (c[u]) {
+      const int64_t pr = (int64_t)(PR)t.r[e[u]].v, ps = (int64_t)(PS)x[u].v;
+      acc.sr += (unsigned long long)pr;
+      acc.ss += (unsigned long long)ps;
+      acc.sx += pair_mix(pr, ps);
+    }
+  }
+  // 3) bag semantics: a chunk with duplicate keys can match again further down
+  if (t.dup) {
+#pragma unroll
+    for (int u = 0; u < U; u++) {
+      for (uint32_t f = c[u] ? t.next[e[u]] : JN_NIL; f != JN_NIL; f = t.next[f]) {
+        if (t.r[f].k == x[u].k) {
+          const int64_t pr = (int64_t)(PR)t.r[f].v, ps = (int64_t)(PS)x[u].v;
+          c[u]++;
+          acc.sr += (unsigned long long)pr;
+          acc.ss += (unsigned long long)ps;
+          acc.sx += pair_mix(pr, ps);
+        }
       }
     }
-    acc.cnt += c[u];
   }
+#pragma unroll
+  for (int u = 0; u < U; u++) acc.cnt += c[u];
   if constexpr (MAT) {
     // positions in (u-major, lane-minor) order inside the warp, warps in order
     // inside the block, one global claim per block per batch
@@ -777,6 +832,7 @@ k_build_probe(JoinArgs a) {
   __shared__ uint32_t s_wsum[JN_CONSUMERS / 32];
   __shared__ unsigned long long s_wbase[JN_CONSUMERS / 32];
   __shared__ unsigned long long s_red[4][JN_THREADS / 32];
+  __shared__ uint32_t s_dup;
 
   const uint32_t nslots = 1u << a.slot_bits;
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
@@ -833,9 +889,21 @@ k_build_probe(JoinArgs a) {
       // ---- build (a11): chained table via atomicExch on the heads
       for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
         s_next[i] = (uint16_t)atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], i);
+      if (threadIdx.x == 0) s_dup = 0;
+      consumer_sync();
+      // duplicate keys share a chain: each tuple looks down its own chain
+      // (short: load factor ~0.5); any equal key switches on bag semantics
+      {
+        bool d = false;
+        for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS) {
+          const auto k = r[i].k;
+          for (uint32_t e = s_next[i]; e != JN_NIL; e = s_next[e]) d |= r[e].k == k;
+        }
+        if (__any_sync(0xffffffffu, d) && lane == 0) s_dup = 1;
+      }
       consumer_sync();
       // ---- probe (a12): stream the S slice
-      const JnTable<KW, PRW> tab{r, s_next, s_head, a.slot_bits};
+      const JnTable<KW, PRW> tab{r, s_next, s_head, a.slot_bits, s_dup != 0};
       uint32_t base = st.s_lo;
       for (; base + JN_U * JN_CONSUMERS <= st.s_hi; base += JN_U * JN_CONSUMERS)
         jn_probe_batch<KW, PRW, PSW, MAT, JN_U>(tab, a, base, st.s_hi, acc, s_wsum, s_wbase);
