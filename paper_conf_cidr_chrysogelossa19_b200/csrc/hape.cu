@@ -289,14 +289,14 @@ static hape_status scatter_v(hape_join* h, const Src& s, SegMap m, BitField bf, 
   static int v = [] { const char* e = getenv("HAPE_SC"); return e ? atoi(e) : -1; }();
   if constexpr (KW + PW <= 8) {
     switch (v) {
-      case 1: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2>>(h, s, m, bf, P, offs, out);
+      case 1: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 2, 3>>(h, s, m, bf, P, offs, out);
       case 2: return scatter_t<KW, PW, AOS, ScCfg<256, 16, 2, 3>>(h, s, m, bf, P, offs, out);
       case 3: return scatter_t<KW, PW, AOS, ScCfg<256, 16, 3, 2>>(h, s, m, bf, P, offs, out);
       case 4: return scatter_t<KW, PW, AOS, ScCfg<512, 16, 2, 1>>(h, s, m, bf, P, offs, out);
       case 5: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 2, 2, true>>(h, s, m, bf, P, offs, out);
       case 6: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2, true>>(h, s, m, bf, P, offs, out);
       case 7: return scatter_t<KW, PW, AOS, ScCfg<256, 16, 2, 2, true>>(h, s, m, bf, P, offs, out);
-      default: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 2, 3>>(h, s, m, bf, P, offs, out);
+      default: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2>>(h, s, m, bf, P, offs, out);
     }
   } else {
     switch (v) {
@@ -526,11 +526,11 @@ extern "C" hape_status hape_exchange_plan(int world_size, int rank, const uint64
 }
 
 static hape_status exchange(hape_join* h, Src in[2], Src out[2]) {
-  const int G = h->cfg.world_size, me = h->cfg.rank;
+  const int G = std::max(1, h->cfg.world_size), me = h->cfg.rank;
   const int kw = key_width(h->cfg);
   const uint32_t g = ceil_log2_u64((uint64_t)G);
   const uint32_t HW = kw * 8;
-  const BitField bf{HW - g, (uint32_t)G - 1};
+  const BitField bf{g ? HW - g : 0u, (uint32_t)G - 1};  // destination = top g bits of h (R14)
   // layout in small: per side hist[G*cps], rowsum[G], and the local bounds block [2][G+1] + gathered [G][2][G+1]
   Carve cv;
   uint32_t cps[2];
@@ -620,7 +620,7 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   CKS(stage_in(h, R, kw, prw, h->stage[0], h->stage[1], &in[0]));
   CKS(stage_in(h, S, kw, psw, h->stage[2], h->stage[3], &in[1]));
   Src loc[2] = {in[0], in[1]};
-  if (world > 1) CKS(exchange(h, in, loc));
+  if (world > 1 || h->comm) CKS(exchange(h, in, loc));
 
   hape_plan pl;
   if (make_plan(h, loc[0].n, loc[1].n, &pl) != HAPE_OK)
@@ -676,7 +676,7 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   CK(h, cudaMemcpyAsync(h->h_res, at<char>(h, L.acc), 4 * 8, cudaMemcpyDeviceToHost, h->stream));
   CK(h, cudaMemcpyAsync(h->h_res + 4, at<char>(h, L.out_ctr), 8, cudaMemcpyDeviceToHost, h->stream));
   CK(h, cudaMemcpyAsync(h->h_res + 5, at<char>(h, L.ctrs), 8, cudaMemcpyDeviceToHost, h->stream));
-  if (world > 1) {
+  if (world > 1 || h->comm) {
     // global result: NCCL allreduce (sum, u64, wrapping) of the four fields
     unsigned long long* acc = at<unsigned long long>(h, L.acc);
     CKN(h, ncclAllReduce(acc, acc, 4, ncclUint64, ncclSum, h->comm, h->stream));
@@ -688,7 +688,7 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   res->local_sum_r = r[1];
   res->local_sum_s = r[2];
   res->local_pair_checksum = r[3];
-  const unsigned long long* g = world > 1 ? r + 6 : r;
+  const unsigned long long* g = (world > 1 || h->comm) ? r + 6 : r;
   res->match_count = g[0];
   res->sum_r_payload = g[1];
   res->sum_s_payload = g[2];

@@ -729,58 +729,31 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
     const uint32_t j = base + u * JN_CONSUMERS + threadIdx.x;
     e0[u] = j < s_hi ? t.head[jn_slot<KW>(x[u].k, t.sbits)] : JN_NIL;
   }
-  // 1) find each tuple's first match: the U chain walks advance together, so
-  //    their dependent shared loads overlap (no warp-wide synchronisation)
-  uint32_t e[U];
-  bool act[U];
-#pragma unroll
-  for (int u = 0; u < U; u++) {
-    e[u] = e0[u];
-    act[u] = e[u] != JN_NIL && t.r[e[u]].k != x[u].k;
-  }
-  while (true) {
-    bool any = false;
-#pragma unroll
-    for (int u = 0; u < U; u++) any |= act[u];
-    if (!any) break;
-#pragma unroll
-    for (int u = 0; u < U; u++) {
-      if (act[u]) {
-        e[u] = t.next[e[u]];
-        act[u] = e[u] != JN_NIL && t.r[e[u]].k != x[u].k;
-      }
-    }
-  }
-  // 2) aggregate the first matches: U independent predicated bodies (the
-  //    64-bit mixing chains interleave)
   uint32_t c[U];
 #pragma unroll
   for (int u = 0; u < U; u++) {
-    c[u] = e[u] != JN_NIL;
-    if (c[u]) {
-      const int64_t pr = (int64_t)(PR)t.r[e[u]].v, ps = (int64_t)(PS)x[u].v;
-      acc.sr += (unsigned long long)pr;
-      acc.ss += (unsigned long long)ps;
-      acc.sx += pair_mix(pr, ps);
-    }
-  }
-  // 3) bag semantics: a chunk with duplicate keys can match again further down
-  if (t.dup) {
-#pragma unroll
-    for (int u = 0; u < U; u++) {
-      for (uint32_t f = c[u] ? t.next[e[u]] : JN_NIL; f != JN_NIL; f = t.next[f]) {
-        if (t.r[f].k == x[u].k) {
-          const int64_t pr = (int64_t)(PR)t.r[f].v, ps = (int64_t)(PS)x[u].v;
-          c[u]++;
-          acc.sr += (unsigned long long)pr;
-          acc.ss += (unsigned long long)ps;
-          acc.sx += pair_mix(pr, ps);
-        }
+    // walk to the next match (divergent, cheap), then run the aggregation
+    // body once per round with every lane that found one (converged).  A
+    // chunk without duplicate keys has at most one match per S tuple, so the
+    // walk stops at the first match.
+    c[u] = 0;
+    uint32_t e = e0[u];
+    while (true) {
+      while (e != JN_NIL && t.r[e].k != x[u].k) e = t.next[e];
+      const bool hit = e != JN_NIL;
+      if (!__any_sync(0xffffffffu, hit)) break;
+      if (hit) {
+        const int64_t pr = (int64_t)(PR)t.r[e].v, ps = (int64_t)(PS)x[u].v;
+        c[u]++;
+        acc.sr += (unsigned long long)pr;
+        acc.ss += (unsigned long long)ps;
+        acc.sx += pair_mix(pr, ps);
+        e = t.next[e];
       }
+      if (!t.dup) break;
     }
+    acc.cnt += c[u];
   }
-#pragma unroll
-  for (int u = 0; u < U; u++) acc.cnt += c[u];
   if constexpr (MAT) {
     // positions in (u-major, lane-minor) order inside the warp, warps in order
     // inside the block, one global claim per block per batch
