@@ -8,7 +8,7 @@ for rep in sys.argv[1:]:
     d = dict(zip(h, v))
     U = dict(zip(h, units))
     SCALE = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9, "nsecond": 1, "usecond": 1e3,
-             "msecond": 1e6, "second": 1e9}
+             "msecond": 1e6, "second": 1e9, "ns": 1, "us": 1e3, "ms": 1e6}
     def g(k):
         try: return float(d[k].replace(",", "")) * SCALE.get(U.get(k, ""), 1)
         except Exception: return float("nan")

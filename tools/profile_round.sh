@@ -1,0 +1,20 @@
+#!/bin/bash
+# Round profiling artefacts (run under gpurun): bench line, clocks, per-launch
+# ncu list of one bench step, and one --set full capture per hot kernel.
+TAG=${1:-r1}
+CFG=${2:-c2}
+mkdir -p gpurun_out
+nvidia-smi --query-gpu=index,clocks.sm,clocks.max.sm,power.draw,clocks_event_reasons.active --format=csv -lms 200 > gpurun_out/clocks_${TAG}_${CFG}.csv &
+SMI=$!
+timeout 600 python bench.py --config $CFG > gpurun_out/bench_${TAG}_${CFG}.json 2> gpurun_out/bench_${TAG}_${CFG}.err
+kill $SMI
+B="python bench.py --config $CFG --steps 1 --warmup 3 --no-e2e --no-cpu-baseline"
+timeout 600 ncu --metrics gpu__time_duration.sum,dram__bytes_read.sum,dram__bytes_write.sum --clock-control none --csv --log-file gpurun_out/launches_${TAG}_${CFG}.csv $B > /dev/null 2>&1
+# per-launch skip counts: 3 warm-up steps precede the profiled one
+NH=$((3*4)); NS=$((3*4)); NB=3
+if [ "$CFG" = "c1" ]; then NH=6; NS=6; fi
+for K in k_hist:$NH k_scatter:$NS k_build_probe:$NB; do
+  N=${K%%:*}; S=${K##*:}
+  timeout 600 ncu --set full --clock-control none --import-source on -k regex:$N -s $S -c 2 -o gpurun_out/full_${TAG}_${CFG}_${N} $B > /dev/null 2>&1
+done
+ls -la gpurun_out
