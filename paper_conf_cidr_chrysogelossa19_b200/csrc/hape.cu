@@ -150,7 +150,8 @@ static int pay_width(hape_dtype t) { return t == HAPE_INT64 ? 8 : 4; }
 
 static uint32_t cps_for(const hape_join* h, uint64_t total, uint32_t nseg) {
   const uint64_t avg = nseg ? (total + nseg - 1) / nseg : total;
-  uint64_t c = (avg + kChunk - 1) / kChunk;
+  static const uint64_t chunk = [] { const char* e = getenv("HAPE_CHUNK"); return e ? (uint64_t)atoll(e) : (uint64_t)kChunk; }();
+  uint64_t c = (avg + chunk - 1) / chunk;
   const uint64_t want_ctas = (uint64_t)h->num_sms * 8;
   if (c * nseg < want_ctas) {
     uint64_t c2 = (want_ctas + nseg - 1) / nseg;
@@ -669,6 +670,8 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   ja.acc = at<unsigned long long>(h, L.acc);
   ja.out_r = mat_r; ja.out_s = mat_s; ja.out_cap = mat ? out->capacity : 0;
   ja.out_ctr = at<unsigned long long>(h, L.out_ctr);
+  static const uint32_t jn_dbg = [] { const char* e = getenv("HAPE_JN_DBG"); return e ? (uint32_t)atoi(e) : 0u; }();
+  ja.dbg = jn_dbg;  // timing experiments only: results are wrong when set
   CKS(launch_join(h, kw, prw, psw, ja, mat, &pl.join_ctas));
 
   mark(h, HAPE_STAGE_FINALIZE);

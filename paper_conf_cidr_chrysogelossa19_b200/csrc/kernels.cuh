@@ -675,6 +675,7 @@ struct JoinArgs {
   uint32_t cap; uint32_t slice; uint32_t slot_bits;
   unsigned long long* acc;                   // [4] count, sum_r, sum_s, checksum
   void* out_r; void* out_s; unsigned long long out_cap; unsigned long long* out_ctr;
+  uint32_t dbg;                              // timing experiments only (HAPE_JN_DBG); 0 in production
 };
 
 struct JnStage {
@@ -860,13 +861,14 @@ k_build_probe(JoinArgs a) {
       const TR* r = reinterpret_cast<const TR*>(ring + bi * RB + st.off);
       consumer_sync();
       // ---- build (a11): chained table via atomicExch on the heads
-      for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
-        s_next[i] = (uint16_t)atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], i);
+      if (!(a.dbg & 4u))
+        for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
+          s_next[i] = (uint16_t)atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], i);
       if (threadIdx.x == 0) s_dup = 0;
       consumer_sync();
       // duplicate keys share a chain: each tuple looks down its own chain
       // (short: load factor ~0.5); any equal key switches on bag semantics
-      {
+      if (!(a.dbg & 8u)) {
         bool d = false;
         for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS) {
           const auto k = r[i].k;
