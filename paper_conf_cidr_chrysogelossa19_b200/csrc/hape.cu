@@ -69,6 +69,11 @@ struct hape_join {
   DevBuf outst[2];        // host-output staging
   DevBuf small;           // histograms, bounds, work list, counters
   unsigned long long* h_res = nullptr;  // pinned: acc[4], out_ctr, (n_items | item_ctr)
+  // cached CUDA graph of the local join sequence (keyed by pointers + sizes)
+  cudaGraphExec_t gexec = nullptr;
+  uintptr_t gkey[14] = {};
+  uint32_t g_launches = 0, g_join_ctas = 0;
+  bool g_ev_used[HAPE_NSTAGES] = {};
   uint32_t* h_bounds = nullptr;         // pinned: gathered device-partition bounds
   size_t h_bounds_cap = 0;
 };
@@ -138,7 +143,12 @@ static hape_status ensure(hape_join* h, DevBuf& b, size_t bytes) {
 }
 
 static void mark(hape_join* h, int stage) {
-  cudaEventRecord(h->ev[stage], h->stream);
+  // inside a stream capture an "external" record becomes a real event-record
+  // node of the graph (a plain record would only express a dependency)
+  cudaStreamCaptureStatus cs = cudaStreamCaptureStatusNone;
+  cudaStreamIsCapturing(h->stream, &cs);
+  if (cs == cudaStreamCaptureStatusActive) cudaEventRecordWithFlags(h->ev[stage], h->stream, cudaEventRecordExternal);
+  else cudaEventRecord(h->ev[stage], h->stream);
   h->ev_used[stage] = true;
 }
 
@@ -646,39 +656,73 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
       mat_s = h->outst[1].p;
     }
   }
-  CK(h, cudaMemsetAsync(at<char>(h, L.zero_lo), 0, L.zero_hi - L.zero_lo, h->stream));
-
-  PassIO io[2];
-  for (int s = 0; s < 2; s++) io[s] = PassIO{loc[s], h->ping[s].p, h->pong[s].p};
-  const void* ft[2];
-  const uint32_t* fb[2];
-  CKS(run_partition_stages(h, pl, L, io, 2, ft, fb));
-
+  // the device-side sequence of one local join; replayed as one CUDA graph
+  // when every pointer and size matches the previous call (launch-latency
+  // bound small joins, BASELINE configs[0])
   const uint32_t Q = 1u << (pl.bits[0] + (pl.passes == 2 ? pl.bits[1] : 0));
   uint32_t* ctrs = at<uint32_t>(h, L.ctrs);  // [0] n_items
-  mark(h, HAPE_STAGE_WORKLIST);
-  k_worklist<<<(Q + WL_THREADS - 1) / WL_THREADS, WL_THREADS, 0, h->stream>>>(fb[0], fb[1], Q, pl.probe_slice,
-                                                                              at<uint2>(h, L.items), ctrs);
-  CK_LAUNCH(h);
-
-  mark(h, HAPE_STAGE_BUILD_PROBE);
-  JoinArgs ja{};
-  ja.rt = ft[0]; ja.st = ft[1];
-  ja.bR = fb[0]; ja.bS = fb[1];
-  ja.items = at<uint2>(h, L.items); ja.n_items = ctrs;
-  ja.cap = pl.build_cap; ja.slice = pl.probe_slice; ja.slot_bits = pl.slot_bits;
-  ja.acc = at<unsigned long long>(h, L.acc);
-  ja.out_r = mat_r; ja.out_s = mat_s; ja.out_cap = mat ? out->capacity : 0;
-  ja.out_ctr = at<unsigned long long>(h, L.out_ctr);
-  static const uint32_t jn_dbg = [] { const char* e = getenv("HAPE_JN_DBG"); return e ? (uint32_t)atoi(e) : 0u; }();
-  ja.dbg = jn_dbg;  // timing experiments only: results are wrong when set
-  CKS(launch_join(h, kw, prw, psw, ja, mat, &pl.join_ctas));
-
-  mark(h, HAPE_STAGE_FINALIZE);
-  // local result: acc[4], out_ctr, ctrs -- contiguous at L.acc (6 x u64)
-  CK(h, cudaMemcpyAsync(h->h_res, at<char>(h, L.acc), 4 * 8, cudaMemcpyDeviceToHost, h->stream));
-  CK(h, cudaMemcpyAsync(h->h_res + 4, at<char>(h, L.out_ctr), 8, cudaMemcpyDeviceToHost, h->stream));
-  CK(h, cudaMemcpyAsync(h->h_res + 5, at<char>(h, L.ctrs), 8, cudaMemcpyDeviceToHost, h->stream));
+  auto enqueue = [&]() -> hape_status {
+    CK(h, cudaMemsetAsync(at<char>(h, L.zero_lo), 0, L.zero_hi - L.zero_lo, h->stream));
+    PassIO io[2];
+    for (int s = 0; s < 2; s++) io[s] = PassIO{loc[s], h->ping[s].p, h->pong[s].p};
+    const void* ft[2];
+    const uint32_t* fb[2];
+    CKS(run_partition_stages(h, pl, L, io, 2, ft, fb));
+    mark(h, HAPE_STAGE_WORKLIST);
+    k_worklist<<<(Q + WL_THREADS - 1) / WL_THREADS, WL_THREADS, 0, h->stream>>>(fb[0], fb[1], Q, pl.probe_slice,
+                                                                                at<uint2>(h, L.items), ctrs);
+    CK_LAUNCH(h);
+    mark(h, HAPE_STAGE_BUILD_PROBE);
+    JoinArgs ja{};
+    ja.rt = ft[0]; ja.st = ft[1];
+    ja.bR = fb[0]; ja.bS = fb[1];
+    ja.items = at<uint2>(h, L.items); ja.n_items = ctrs;
+    ja.cap = pl.build_cap; ja.slice = pl.probe_slice; ja.slot_bits = pl.slot_bits;
+    ja.acc = at<unsigned long long>(h, L.acc);
+    ja.out_r = mat_r; ja.out_s = mat_s; ja.out_cap = mat ? out->capacity : 0;
+    ja.out_ctr = at<unsigned long long>(h, L.out_ctr);
+    static const uint32_t jn_dbg = [] { const char* e = getenv("HAPE_JN_DBG"); return e ? (uint32_t)atoi(e) : 0u; }();
+    ja.dbg = jn_dbg;  // timing experiments only: results are wrong when set
+    CKS(launch_join(h, kw, prw, psw, ja, mat, &pl.join_ctas));
+    mark(h, HAPE_STAGE_FINALIZE);
+    // local result: acc[4], out_ctr, ctrs
+    CK(h, cudaMemcpyAsync(h->h_res, at<char>(h, L.acc), 4 * 8, cudaMemcpyDeviceToHost, h->stream));
+    CK(h, cudaMemcpyAsync(h->h_res + 4, at<char>(h, L.out_ctr), 8, cudaMemcpyDeviceToHost, h->stream));
+    CK(h, cudaMemcpyAsync(h->h_res + 5, at<char>(h, L.ctrs), 8, cudaMemcpyDeviceToHost, h->stream));
+    return HAPE_OK;
+  };
+  static const bool no_graph = getenv("HAPE_NO_GRAPH") != nullptr;
+  const bool graphable = !no_graph && world == 1 && !h->comm && R->mem == HAPE_MEM_DEVICE &&
+                         S->mem == HAPE_MEM_DEVICE && (!mat || out->mem == HAPE_MEM_DEVICE);
+  if (graphable) {
+    const uintptr_t key[] = {(uintptr_t)R->key, (uintptr_t)R->payload, (uintptr_t)R->n, (uintptr_t)S->key,
+                             (uintptr_t)S->payload, (uintptr_t)S->n, (uintptr_t)mat_r, (uintptr_t)mat_s,
+                             (uintptr_t)(mat ? out->capacity : 0), (uintptr_t)h->small.p, (uintptr_t)h->ping[0].p,
+                             (uintptr_t)h->ping[1].p, (uintptr_t)h->pong[0].p, (uintptr_t)h->pong[1].p};
+    static_assert(sizeof key == sizeof h->gkey, "graph key size");
+    if (!h->gexec || memcmp(key, h->gkey, sizeof key) != 0) {
+      if (h->gexec) { cudaGraphExecDestroy(h->gexec); h->gexec = nullptr; }
+      cudaGraph_t g = nullptr;
+      CK(h, cudaStreamBeginCapture(h->stream, cudaStreamCaptureModeThreadLocal));
+      const hape_status st = enqueue();
+      const cudaError_t ce = cudaStreamEndCapture(h->stream, &g);
+      if (st != HAPE_OK) { if (g) cudaGraphDestroy(g); return st; }
+      CK(h, ce);
+      const cudaError_t ie = cudaGraphInstantiate(&h->gexec, g, 0);
+      cudaGraphDestroy(g);
+      CK(h, ie);
+      memcpy(h->gkey, key, sizeof key);
+      h->g_launches = h->launches;
+      memcpy(h->g_ev_used, h->ev_used, sizeof h->g_ev_used);
+      h->g_join_ctas = pl.join_ctas;
+    }
+    CK(h, cudaGraphLaunch(h->gexec, h->stream));
+    h->launches = h->g_launches;
+    for (int i = HAPE_STAGE_HIST1; i < HAPE_STAGE_TOTAL; i++) h->ev_used[i] = h->g_ev_used[i];
+    pl.join_ctas = h->g_join_ctas;
+  } else {
+    CKS(enqueue());
+  }
   if (world > 1 || h->comm) {
     // global result: NCCL allreduce (sum, u64, wrapping) of the four fields
     unsigned long long* acc = at<unsigned long long>(h, L.acc);
@@ -822,6 +866,7 @@ hape_status hape_join_destroy(hape_join* h) {
       if (g[i].p) cudaFree(g[i].p);
   for (auto& b : h->outst)
     if (b.p) cudaFree(b.p);
+  if (h->gexec) cudaGraphExecDestroy(h->gexec);
   if (h->small.p) cudaFree(h->small.p);
   if (h->h_res) cudaFreeHost(h->h_res);
   if (h->h_bounds) cudaFreeHost(h->h_bounds);
