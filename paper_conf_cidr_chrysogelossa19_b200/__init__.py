@@ -99,8 +99,12 @@ class RadixJoin:
         cfg.max_r, cfg.max_s = max_r, max_s
         cfg.world_size, cfg.rank = world_size, rank
         cfg.nccl_comm = nccl_comm.value if isinstance(nccl_comm, ctypes.c_void_p) else nccl_comm
-        if stream is not None:
-            cfg.stream = stream.cuda_stream if hasattr(stream, "cuda_stream") else int(stream)
+        # the library enqueues on the caller's stream (inputs must be ready on
+        # it): default to torch's current stream on the device
+        if stream is None:
+            stream = torch.cuda.current_stream(device)
+        cfg.stream = stream.cuda_stream if hasattr(stream, "cuda_stream") else int(stream)
+        self._stream_handle = cfg.stream
         self.cfg = cfg
         st, h = hape_join_create(cfg)
         if st != HAPE_OK:
@@ -134,7 +138,16 @@ class RadixJoin:
             raise HapeError(st, hape_last_error(self._h))
         return p
 
+    def _order_inputs(self):
+        """Inputs produced on another torch stream must be complete before the
+        library's stream reads them (the ABI leaves ordering to the caller)."""
+        import torch
+        cur = torch.cuda.current_stream(self.cfg.device)
+        if cur.cuda_stream != self._stream_handle:
+            cur.synchronize()
+
     def join(self, rk, rp, sk, sp, out_r=None, out_s=None, raise_on_capacity: bool = True) -> JoinResult:
+        self._order_inputs()
         R = _rel(rk, rp)
         S = _rel(sk, sp)
         out = None
@@ -162,6 +175,7 @@ class RadixJoin:
         """Run the planned radix passes on one relation; returns
         (partitioned keys, partitioned payloads, bounds[int64], plan)."""
         import torch
+        self._order_inputs()
         rel = _rel(key, pay)
         dev = torch.device("cuda", self.cfg.device)
         ok = torch.empty_like(key, device=dev)

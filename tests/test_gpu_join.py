@@ -250,3 +250,52 @@ def test_identity_partitions_equal_size():
     wl = datagen.make("c1", n_r=n, n_s=n)
     res = j.join(cuda(wl.R.key), cuda(wl.R.payload), cuda(wl.S.key), cuda(wl.S.payload))
     check(res, provenance.expected_from_workload(wl))
+
+
+# ---- BASELINE full sizes, in the launch configuration bench.py times --------
+@pytest.mark.slow
+def test_c2_full_size_vs_oracle():
+    # configs[1]: |R|=|S|=2^27 int32, 2-pass; the oracle's sort-merge (~15 s)
+    # and the generator provenance both check the device result
+    wl = datagen.make("c2", backend="torch", device="cuda")
+    j = RadixJoin(key_dtype=torch.int32, max_r=1 << 27, max_s=1 << 27)
+    res = j.join(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload)
+    rk, rp, sk, sp = (x.cpu().numpy() for x in (wl.R.key, wl.R.payload, wl.S.key, wl.S.payload))
+    want = oracle_res(rk, rp, sk, sp)
+    check(res, want)
+    assert res.passes == 2 and res.bits == (8, 8)
+    prov = provenance.expected_pkfk(rp[wl.idx.cpu().numpy()], sp)
+    assert prov == want
+
+
+@pytest.mark.slow
+def test_c3_full_size_pairs_vs_provenance():
+    # configs[2]: |R|=2^27, |S|=2^30 int64, 2^30 materialised pairs.  Count,
+    # sums and checksum vs the provenance closed forms (oracle/provenance.py);
+    # the pair multiset vs provenance by a sorted compare on the device.
+    wl = datagen.make("c3", backend="torch", device="cuda")
+    n = wl.S.key.shape[0]
+    out_r = torch.empty(n, dtype=torch.int64, device="cuda")
+    out_s = torch.empty(n, dtype=torch.int64, device="cuda")
+    j = RadixJoin(key_dtype=torch.int64, max_r=1 << 27, max_s=1 << 30)
+    res = j.join(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload, out_r, out_s)
+    exp_r = wl.R.payload[wl.idx]
+    want = provenance.expected_pkfk(exp_r.cpu().numpy(), wl.S.payload.cpu().numpy())
+    check(res, want)
+    assert res.n_written == n
+    # every S payload is unique (sm() is a bijection), so sorting by s orders both sides
+    o_got = torch.argsort(out_s)
+    o_exp = torch.argsort(wl.S.payload)
+    assert torch.equal(out_s[o_got], wl.S.payload[o_exp])
+    assert torch.equal(out_r[o_got], exp_r[o_exp])
+
+
+@pytest.mark.parametrize("theta", [0.5, 1.0])
+def test_zipf_skew_vs_oracle(theta):
+    # C5's skew recipe at one-GPU scale: the hottest key spans many S slices
+    wl = datagen.make("c5", n_r=1 << 20, n_s=1 << 22, theta=theta)
+    want = oracle_res(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload)
+    res = joiner(torch.int32).join(cuda(wl.R.key), cuda(wl.R.payload), cuda(wl.S.key), cuda(wl.S.payload))
+    check(res, want)
+    if theta == 1.0:
+        assert res.n_items > res.n_partitions  # the hot co-partitions were split into S slices
