@@ -55,6 +55,8 @@ struct hape_join {
   int num_sms = 148;
   cudaStream_t stream = nullptr;
   bool own_stream = false;
+  cudaStream_t copy_stream = nullptr;   // host-input S transfer (overlaps R's passes)
+  cudaEvent_t ev_copy = nullptr;
   ncclComm_t comm = nullptr;
   std::string err;
   cudaEvent_t ev[HAPE_NSTAGES + 1] = {};
@@ -445,46 +447,69 @@ struct PassIO {
   void* p2;     // pass-2 output tuples
 };
 
+// side1_ready != nullptr: host-resident inputs whose S copy is still in
+// flight on the copy stream -- run all of R's passes first (overlapping the S
+// transfer), then wait for the copy and run S's.  Stage marks then cover
+// both sides' work in sequence.
 static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const CallLayout& L, PassIO io[2],
-                                        int nside, const void** fin, const uint32_t** fin_bounds) {
+                                        int nside, const void** fin, const uint32_t** fin_bounds,
+                                        cudaEvent_t side1_ready = nullptr) {
   const int kw = key_width(h->cfg);
   const uint32_t P1 = 1u << pl.bits[0], P2 = 1u << pl.bits[1];
   const BitField bf1{0u, P1 - 1}, bf2{pl.bits[0], P2 - 1};
   SegMap m1[2], m2[2];
+  Src s2[2];
   for (int s = 0; s < nside; s++) {
     m1[s] = SegMap{nullptr, 1u, L.side[s].cps1, io[s].in.n};
     if (pl.passes == 2) m2[s] = SegMap{at<uint32_t>(h, L.side[s].bounds1), P1, L.side[s].cps2, io[s].in.n};
+    s2[s] = Src{PartIn{nullptr, nullptr, io[s].p1}, true, io[s].in.n, io[s].in.pw};
   }
-  mark(h, HAPE_STAGE_HIST1);
-  for (int s = 0; s < nside; s++)
-    CKS(launch_hist(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1)));
-  mark(h, HAPE_STAGE_SCAN1);
-  for (int s = 0; s < nside; s++)
-    CKS(launch_scan(h, m1[s], P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1),
-                    at<uint32_t>(h, L.side[s].bounds1)));
-  mark(h, HAPE_STAGE_SCATTER1);
-  for (int s = 0; s < nside; s++)
-    CKS(launch_scatter(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), io[s].p1));
-  for (int s = 0; s < nside; s++) {
-    fin[s] = io[s].p1;
-    fin_bounds[s] = at<uint32_t>(h, L.side[s].bounds1);
-  }
-  if (pl.passes == 2) {
-    Src s2[2];
-    for (int s = 0; s < nside; s++) s2[s] = Src{PartIn{nullptr, nullptr, io[s].p1}, true, io[s].in.n, io[s].in.pw};
-    mark(h, HAPE_STAGE_HIST2);
-    for (int s = 0; s < nside; s++)
-      CKS(launch_hist(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), at<uint32_t>(h, L.side[s].rowsum2)));
-    mark(h, HAPE_STAGE_SCAN2);
-    for (int s = 0; s < nside; s++)
-      CKS(launch_scan(h, m2[s], P2, at<uint32_t>(h, L.side[s].hist2), at<uint32_t>(h, L.side[s].rowsum2),
-                      at<uint32_t>(h, L.side[s].bounds2)));
-    mark(h, HAPE_STAGE_SCATTER2);
+  auto hist1 = [&](int s) {
+    return launch_hist(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1));
+  };
+  auto scan1 = [&](int s) {
+    return launch_scan(h, m1[s], P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1),
+                       at<uint32_t>(h, L.side[s].bounds1));
+  };
+  auto scatter1 = [&](int s) {
+    return launch_scatter(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), io[s].p1);
+  };
+  auto hist2 = [&](int s) {
+    return launch_hist(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), at<uint32_t>(h, L.side[s].rowsum2));
+  };
+  auto scan2 = [&](int s) {
+    return launch_scan(h, m2[s], P2, at<uint32_t>(h, L.side[s].hist2), at<uint32_t>(h, L.side[s].rowsum2),
+                       at<uint32_t>(h, L.side[s].bounds2));
+  };
+  auto scatter2 = [&](int s) {
+    return launch_scatter(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), io[s].p2);
+  };
+  if (side1_ready) {
     for (int s = 0; s < nside; s++) {
-      CKS(launch_scatter(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), io[s].p2));
-      fin[s] = io[s].p2;
-      fin_bounds[s] = at<uint32_t>(h, L.side[s].bounds2);
+      if (s == 1) CK(h, cudaStreamWaitEvent(h->stream, side1_ready, 0));
+      if (s == 0) mark(h, HAPE_STAGE_HIST1);
+      CKS(hist1(s)); CKS(scan1(s)); CKS(scatter1(s));
+      if (pl.passes == 2) { CKS(hist2(s)); CKS(scan2(s)); CKS(scatter2(s)); }
     }
+  } else {
+    mark(h, HAPE_STAGE_HIST1);
+    for (int s = 0; s < nside; s++) CKS(hist1(s));
+    mark(h, HAPE_STAGE_SCAN1);
+    for (int s = 0; s < nside; s++) CKS(scan1(s));
+    mark(h, HAPE_STAGE_SCATTER1);
+    for (int s = 0; s < nside; s++) CKS(scatter1(s));
+    if (pl.passes == 2) {
+      mark(h, HAPE_STAGE_HIST2);
+      for (int s = 0; s < nside; s++) CKS(hist2(s));
+      mark(h, HAPE_STAGE_SCAN2);
+      for (int s = 0; s < nside; s++) CKS(scan2(s));
+      mark(h, HAPE_STAGE_SCATTER2);
+      for (int s = 0; s < nside; s++) CKS(scatter2(s));
+    }
+  }
+  for (int s = 0; s < nside; s++) {
+    fin[s] = pl.passes == 2 ? io[s].p2 : io[s].p1;
+    fin_bounds[s] = at<uint32_t>(h, pl.passes == 2 ? L.side[s].bounds2 : L.side[s].bounds1);
   }
   return HAPE_OK;
 }
@@ -504,7 +529,8 @@ static hape_status check_rel(hape_join* h, const hape_relation* r, int kw, int p
 }
 
 static hape_status stage_in(hape_join* h, const hape_relation* r, int kw, int pw, DevBuf& bk, DevBuf& bp,
-                            Src* out) {
+                            Src* out, cudaStream_t st = nullptr) {
+  if (!st) st = h->stream;
   out->n = (uint32_t)r->n;
   out->pw = pw;
   out->aos = false;
@@ -514,8 +540,8 @@ static hape_status stage_in(hape_join* h, const hape_relation* r, int kw, int pw
   }
   CKS(ensure(h, bk, r->n * kw));
   CKS(ensure(h, bp, r->n * pw));
-  CK(h, cudaMemcpyAsync(bk.p, r->key, r->n * kw, cudaMemcpyHostToDevice, h->stream));
-  CK(h, cudaMemcpyAsync(bp.p, r->payload, r->n * pw, cudaMemcpyHostToDevice, h->stream));
+  CK(h, cudaMemcpyAsync(bk.p, r->key, r->n * kw, cudaMemcpyHostToDevice, st));
+  CK(h, cudaMemcpyAsync(bp.p, r->payload, r->n * pw, cudaMemcpyHostToDevice, st));
   out->in = PartIn{bk.p, bp.p, nullptr};
   return HAPE_OK;
 }
@@ -628,8 +654,18 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   mark(h, HAPE_STAGE_TOTAL);
   mark(h, HAPE_STAGE_H2D);
   Src in[2];
+  // host-resident S (single GPU): copy it on the copy stream, overlapping the
+  // R copy's successors (R's radix passes run while S is in flight)
+  const bool overlap = world == 1 && !h->comm && S->mem == HAPE_MEM_HOST && S->n > 0;
   CKS(stage_in(h, R, kw, prw, h->stage[0], h->stage[1], &in[0]));
-  CKS(stage_in(h, S, kw, psw, h->stage[2], h->stage[3], &in[1]));
+  if (overlap) {
+    CK(h, cudaEventRecord(h->ev_copy, h->stream));          // S staging buffers are free
+    CK(h, cudaStreamWaitEvent(h->copy_stream, h->ev_copy, 0));
+    CKS(stage_in(h, S, kw, psw, h->stage[2], h->stage[3], &in[1], h->copy_stream));
+    CK(h, cudaEventRecord(h->ev_copy, h->copy_stream));
+  } else {
+    CKS(stage_in(h, S, kw, psw, h->stage[2], h->stage[3], &in[1]));
+  }
   Src loc[2] = {in[0], in[1]};
   if (world > 1 || h->comm) CKS(exchange(h, in, loc));
 
@@ -667,7 +703,7 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
     for (int s = 0; s < 2; s++) io[s] = PassIO{loc[s], h->ping[s].p, h->pong[s].p};
     const void* ft[2];
     const uint32_t* fb[2];
-    CKS(run_partition_stages(h, pl, L, io, 2, ft, fb));
+    CKS(run_partition_stages(h, pl, L, io, 2, ft, fb, overlap ? h->ev_copy : nullptr));
     mark(h, HAPE_STAGE_WORKLIST);
     k_worklist<<<(Q + WL_THREADS - 1) / WL_THREADS, WL_THREADS, 0, h->stream>>>(fb[0], fb[1], Q, pl.probe_slice,
                                                                                 at<uint2>(h, L.items), ctrs);
@@ -835,6 +871,8 @@ hape_status hape_join_create(const hape_join_config* cfg, hape_join** out_handle
     }
     for (auto& e : h->ev)
       if (cudaEventCreate(&e) != cudaSuccess) { st = HAPE_ERR_CUDA; break; }
+    if (cudaStreamCreateWithFlags(&h->copy_stream, cudaStreamNonBlocking) != cudaSuccess ||
+        cudaEventCreateWithFlags(&h->ev_copy, cudaEventDisableTiming) != cudaSuccess) { st = HAPE_ERR_CUDA; break; }
     if (st != HAPE_OK) break;
     if (cudaMallocHost(&h->h_res, 16 * sizeof(unsigned long long)) != cudaSuccess) { st = HAPE_ERR_OOM; break; }
     if (cfg->max_r || cfg->max_s) {
@@ -872,6 +910,8 @@ hape_status hape_join_destroy(hape_join* h) {
   if (h->h_bounds) cudaFreeHost(h->h_bounds);
   for (auto& e : h->ev)
     if (e) cudaEventDestroy(e);
+  if (h->copy_stream) { cudaStreamSynchronize(h->copy_stream); cudaStreamDestroy(h->copy_stream); }
+  if (h->ev_copy) cudaEventDestroy(h->ev_copy);
   if (h->own_stream && h->stream) cudaStreamDestroy(h->stream);
   (void)cudaGetLastError();
   delete h;
