@@ -172,6 +172,8 @@ def main():
     ap.add_argument("--verify", action="store_true", help="check the result against generator provenance")
     ap.add_argument("--bits", default="0,0", help="radix bits per pass (0 = auto; tuning only)")
     ap.add_argument("--passes", type=int, default=0, help="radix passes (0 = auto; tuning only)")
+    ap.add_argument("--exchange", action="store_true",
+                    help="at N=1, run the device-partition + NCCL exchange path through a 1-rank communicator")
     args = ap.parse_args()
     if args.impl == "reference":
         return run_reference(args)
@@ -200,9 +202,10 @@ def main():
     materialize = cfg == "c3"
 
     comm = None
-    if world > 1:
+    if world > 1 or args.exchange:
         uid = [_lib.hape_nccl_unique_id() if rank == 0 else None]
-        dist.broadcast_object_list(uid, src=0)
+        if world > 1:
+            dist.broadcast_object_list(uid, src=0)
         st, comm = _lib.hape_nccl_comm_init(uid[0], world, rank, local)
         assert st == 0, f"nccl comm init failed: {st}"
     stream = torch.cuda.current_stream()
@@ -291,7 +294,12 @@ def main():
     except Exception:
         pass
     achieved = per_stage[dom]["GB/s"]
-    alg_total = sum(alg[k] for k in alg if k != "devpart") + (alg["devpart"] if world > 1 else 0)
+    alg_total = sum(alg[k] for k in alg if k != "devpart") + (alg["devpart"] if (world > 1 or args.exchange) else 0)
+    if stage_avg.get("exchange", 0) > 0:
+        xb = t * (nr_loc + ns_loc)  # every local tuple leaves through the exchange (incl. the self segment)
+        per_stage["exchange"] = {"ms": round(stage_avg["exchange"], 4), "bytes_sent": xb,
+                                 "GB/s": round(xb / (stage_avg["exchange"] / 1000.0) / 1e9, 1),
+                                 "bound": "nvlink (NCCL all-to-allv)"}
     roofline = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
                 "frac": round(achieved / peak, 4), "traffic": traffic, "kernel": kernel_name[dom],
                 "peak_source": peak_src,
@@ -338,7 +346,8 @@ def main():
             "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "weak",
             "vs_baseline": None, "dtype": "int32" if wl.key_bits == 32 else "int64",
             "data": "synthetic (datagen counter-based recipe, generated on device)",
-            "config": {"workload": f"{cfg}: {CONFIG_TEXT[cfg]}" + (f"; {world} ranks x shard" if world > 1 else ""),
+            "config": {"workload": f"{cfg}: {CONFIG_TEXT[cfg]}" + (f"; {world} ranks x shard" if world > 1 else "")
+                       + ("; through the 1-rank NCCL exchange path" if (args.exchange and world == 1) else ""),
                        "n_r": n_r, "n_s": n_s, "per_rank_r": nr_loc, "per_rank_s": ns_loc,
                        "passes": res.passes, "bits": list(res.bits), "n_items": res.n_items,
                        "materialize": materialize,
