@@ -172,6 +172,8 @@ def main():
     ap.add_argument("--verify", action="store_true", help="check the result against generator provenance")
     ap.add_argument("--bits", default="0,0", help="radix bits per pass (0 = auto; tuning only)")
     ap.add_argument("--passes", type=int, default=0, help="radix passes (0 = auto; tuning only)")
+    ap.add_argument("--bag", action="store_true",
+                    help="do not declare R's keys unique (HAPE_FLAG_R_UNIQUE): full bag-semantics probe")
     ap.add_argument("--exchange", action="store_true",
                     help="at N=1, run the device-partition + NCCL exchange path through a 1-rank communicator")
     args = ap.parse_args()
@@ -212,6 +214,7 @@ def main():
     j = RadixJoin(key_dtype=kdt, r_payload_dtype=pdt, s_payload_dtype=pdt, device=local,
                   max_r=nr_loc, max_s=ns_loc, world_size=world, rank=rank,
                   radix_passes=args.passes, radix_bits=tuple(int(x) for x in args.bits.split(",")),
+                  r_unique=not args.bag,
                   nccl_comm=comm, stream=stream)
     out_r = out_s = None
     if materialize:
@@ -350,6 +353,7 @@ def main():
                        + ("; through the 1-rank NCCL exchange path" if (args.exchange and world == 1) else ""),
                        "n_r": n_r, "n_s": n_s, "per_rank_r": nr_loc, "per_rank_s": ns_loc,
                        "passes": res.passes, "bits": list(res.bits), "n_items": res.n_items,
+                       "r_unique_declared": not args.bag,
                        "materialize": materialize,
                        "l2": "inputs and workspace (>=2 GiB per step) exceed the 126 MB L2; no flush needed",
                        "parallelism": f"hash-sharded x{world}" if world > 1 else "1 GPU"},

@@ -26,6 +26,7 @@ HAPE_PART_HASH = 0
 HAPE_PART_IDENTITY = 1
 HAPE_MEM_DEVICE = 0
 HAPE_MEM_HOST = 1
+HAPE_FLAG_R_UNIQUE = 1
 
 STAGES = ["h2d", "devpart", "exchange", "hist1", "scan1", "scatter1", "hist2", "scan2",
           "scatter2", "worklist", "build_probe", "finalize", "total"]

@@ -719,6 +719,7 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
     ja.out_ctr = at<unsigned long long>(h, L.out_ctr);
     static const uint32_t jn_dbg = [] { const char* e = getenv("HAPE_JN_DBG"); return e ? (uint32_t)atoi(e) : 0u; }();
     ja.dbg = jn_dbg;  // timing experiments only: results are wrong when set
+    ja.r_unique = (c.flags & HAPE_FLAG_R_UNIQUE) ? 1u : 0u;
     CKS(launch_join(h, kw, prw, psw, ja, mat, &pl.join_ctas));
     mark(h, HAPE_STAGE_FINALIZE);
     // local result: acc[4], out_ctr, ctrs
@@ -850,6 +851,7 @@ hape_status hape_join_create(const hape_join_config* cfg, hape_join** out_handle
   if (cfg->rank < 0 || cfg->rank >= world) return HAPE_ERR_INVALID_ARG;
   if (world > 1 && !cfg->nccl_comm) return HAPE_ERR_INVALID_ARG;
   if (cfg->device < 0) return HAPE_ERR_INVALID_ARG;
+  if (cfg->flags & ~HAPE_FLAG_R_UNIQUE) return HAPE_ERR_INVALID_ARG;
   int ndev = 0;
   if (cudaGetDeviceCount(&ndev) != cudaSuccess || cfg->device >= ndev) {
     (void)cudaGetLastError();

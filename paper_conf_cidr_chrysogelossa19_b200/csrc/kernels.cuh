@@ -676,6 +676,7 @@ struct JoinArgs {
   unsigned long long* acc;                   // [4] count, sum_r, sum_s, checksum
   void* out_r; void* out_s; unsigned long long out_cap; unsigned long long* out_ctr;
   uint32_t dbg;                              // timing experiments only (HAPE_JN_DBG); 0 in production
+  uint32_t r_unique;                         // caller guarantees unique R keys (HAPE_FLAG_R_UNIQUE)
 };
 
 struct JnStage {
@@ -866,16 +867,9 @@ k_build_probe(JoinArgs a) {
           s_next[i] = (uint16_t)atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], i);
       if (threadIdx.x == 0) s_dup = 0;
       consumer_sync();
-      // duplicate keys share a chain: each tuple looks down its own chain
-      // (short: load factor ~0.5); any equal key switches on bag semantics
-      if (!(a.dbg & 8u)) {
-        bool d = false;
-        for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS) {
-          const auto k = r[i].k;
-          for (uint32_t e = s_next[i]; e != JN_NIL; e = s_next[e]) d |= r[e].k == k;
-        }
-        if (__any_sync(0xffffffffu, d) && lane == 0) s_dup = 1;
-      }
+      // bag semantics walk every chain to its end; a caller-declared unique
+      // build side (HAPE_FLAG_R_UNIQUE, a primary key) stops at the first match
+      if (threadIdx.x == 0) s_dup = a.r_unique ? 0u : 1u;
       consumer_sync();
       // ---- probe (a12): stream the S slice
       const JnTable<KW, PRW> tab{r, s_next, s_head, a.slot_bits, s_dup != 0};

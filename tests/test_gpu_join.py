@@ -96,6 +96,24 @@ def test_config_recipes_vs_oracle(cfg, nr, ns):
     assert res.match_count == ns  # closed form (P793-794)
 
 
+@pytest.mark.parametrize("cfg,nr,ns", [("c1", 1 << 18, 1 << 18), ("c3", 1 << 16, 1 << 19),
+                                       ("c5", 1 << 17, 1 << 19), ("c2", 100_003, 200_011)])
+def test_declared_unique_build_side_vs_oracle(cfg, nr, ns):
+    # HAPE_FLAG_R_UNIQUE (R is a primary key in every BASELINE recipe): the
+    # probe stops at the first match; results must not change
+    wl = datagen.make(cfg, n_r=nr, n_s=ns)
+    kdt = DT[wl.key_bits]
+    want = oracle_res(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload, materialize=True)
+    n = want["count"]
+    out_r = torch.empty(n, dtype=kdt, device="cuda")
+    out_s = torch.empty(n, dtype=kdt, device="cuda")
+    res = joiner(kdt, r_unique=True).join(cuda(wl.R.key), cuda(wl.R.payload), cuda(wl.S.key), cuda(wl.S.payload),
+                                          out_r, out_s)
+    check(res, want)
+    a, b = sorted_pairs(out_r, out_s)
+    assert np.array_equal(a, want["pairs"][0]) and np.array_equal(b, want["pairs"][1])
+
+
 def test_c1_full_with_pairs_vs_oracle():
     wl = datagen.make("c1")
     want = oracle_res(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload, materialize=True)
@@ -258,7 +276,7 @@ def test_c2_full_size_vs_oracle():
     # configs[1]: |R|=|S|=2^27 int32, 2-pass; the oracle's sort-merge (~15 s)
     # and the generator provenance both check the device result
     wl = datagen.make("c2", backend="torch", device="cuda")
-    j = RadixJoin(key_dtype=torch.int32, max_r=1 << 27, max_s=1 << 27)
+    j = RadixJoin(key_dtype=torch.int32, max_r=1 << 27, max_s=1 << 27, r_unique=True)  # as bench.py
     res = j.join(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload)
     rk, rp, sk, sp = (x.cpu().numpy() for x in (wl.R.key, wl.R.payload, wl.S.key, wl.S.payload))
     want = oracle_res(rk, rp, sk, sp)
@@ -277,7 +295,7 @@ def test_c3_full_size_pairs_vs_provenance():
     n = wl.S.key.shape[0]
     out_r = torch.empty(n, dtype=torch.int64, device="cuda")
     out_s = torch.empty(n, dtype=torch.int64, device="cuda")
-    j = RadixJoin(key_dtype=torch.int64, max_r=1 << 27, max_s=1 << 30)
+    j = RadixJoin(key_dtype=torch.int64, max_r=1 << 27, max_s=1 << 30, r_unique=True)
     res = j.join(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload, out_r, out_s)
     exp_r = wl.R.payload[wl.idx]
     want = provenance.expected_pkfk(exp_r.cpu().numpy(), wl.S.payload.cpu().numpy())
