@@ -172,6 +172,7 @@ def main():
     ap.add_argument("--verify", action="store_true", help="check the result against generator provenance")
     ap.add_argument("--bits", default="0,0", help="radix bits per pass (0 = auto; tuning only)")
     ap.add_argument("--passes", type=int, default=0, help="radix passes (0 = auto; tuning only)")
+    ap.add_argument("--no-mat", action="store_true", help="c3 without materialised pairs (diagnostics)")
     ap.add_argument("--bag", action="store_true",
                     help="do not declare R's keys unique (HAPE_FLAG_R_UNIQUE): full bag-semantics probe")
     ap.add_argument("--exchange", action="store_true",
@@ -201,7 +202,7 @@ def main():
     pdt = torch.int32 if wl.pay_bits == 32 else torch.int64
     rk, rp, sk, sp = (x.contiguous() for x in (wl.R.key, wl.R.payload, wl.S.key, wl.S.payload))
     nr_loc, ns_loc = rk.shape[0], sk.shape[0]
-    materialize = cfg == "c3"
+    materialize = cfg == "c3" and not args.no_mat
 
     comm = None
     if world > 1 or args.exchange:

@@ -731,7 +731,7 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
     const uint32_t j = base + u * JN_CONSUMERS + threadIdx.x;
     e0[u] = j < s_hi ? t.head[jn_slot<KW>(x[u].k, t.sbits)] : JN_NIL;
   }
-  uint32_t c[U];
+  uint32_t c[U], m[U];
 #pragma unroll
   for (int u = 0; u < U; u++) {
     // walk to the next match (divergent, cheap), then run the aggregation
@@ -739,6 +739,7 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
     // chunk without duplicate keys has at most one match per S tuple, so the
     // walk stops at the first match.
     c[u] = 0;
+    m[u] = JN_NIL;
     uint32_t e = e0[u];
     while (true) {
       while (e != JN_NIL && t.r[e].k != x[u].k) e = t.next[e];
@@ -746,6 +747,7 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
       if (!__any_sync(0xffffffffu, hit)) break;
       if (hit) {
         const int64_t pr = (int64_t)(PR)t.r[e].v, ps = (int64_t)(PS)x[u].v;
+        if (MAT && c[u] == 0) m[u] = e;
         c[u]++;
         acc.sr += (unsigned long long)pr;
         acc.ss += (unsigned long long)ps;
@@ -758,24 +760,52 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
   }
   if constexpr (MAT) {
     // positions in (u-major, lane-minor) order inside the warp, warps in order
-    // inside the block, one global claim per block per batch
+    // inside the block, one global claim per block per batch.  With a unique
+    // build side every count is 0/1: a ballot gives the positions and the
+    // recorded match is written without walking the chain again.
     uint32_t incl[U], before[U], wtot = 0;
+    if (!t.dup) {
+      const uint32_t lt = (1u << lane) - 1u;
 #pragma unroll
-    for (int u = 0; u < U; u++) {
-      incl[u] = warp_incl_scan(c[u]);
-      before[u] = wtot;
-      wtot += __shfl_sync(0xffffffffu, incl[u], 31);
+      for (int u = 0; u < U; u++) {
+        const uint32_t mk = __ballot_sync(0xffffffffu, c[u] != 0);
+        before[u] = wtot;
+        incl[u] = __popc(mk & lt) + c[u];
+        wtot += __popc(mk);
+      }
+    } else {
+#pragma unroll
+      for (int u = 0; u < U; u++) {
+        incl[u] = warp_incl_scan(c[u]);
+        before[u] = wtot;
+        wtot += __shfl_sync(0xffffffffu, incl[u], 31);
+      }
     }
     if (lane == 0) s_wsum[warp] = wtot;
     consumer_sync();
-    if (threadIdx.x == 0) {
-      unsigned long long run = 0;
-      for (int w = 0; w < JN_CONSUMERS / 32; w++) { s_wbase[w] = run; run += s_wsum[w]; }
-      const unsigned long long g = run ? atomicAdd(a.out_ctr, run) : 0ull;
-      for (int w = 0; w < JN_CONSUMERS / 32; w++) s_wbase[w] += g;
+    if (warp == 0) {
+      const uint32_t v = lane < JN_CONSUMERS / 32 ? s_wsum[lane] : 0u;
+      const uint32_t inc = warp_incl_scan(v);
+      const uint32_t tot = __shfl_sync(0xffffffffu, inc, 31);
+      unsigned long long g = 0;
+      if (lane == 0 && tot) g = atomicAdd(a.out_ctr, (unsigned long long)tot);
+      g = __shfl_sync(0xffffffffu, g, 0);
+      if (lane < JN_CONSUMERS / 32) s_wbase[lane] = g + inc - v;
     }
     consumer_sync();
     const unsigned long long wb = s_wbase[warp];
+    if (!t.dup) {
+#pragma unroll
+      for (int u = 0; u < U; u++) {
+        if (!c[u]) continue;
+        const unsigned long long pos = wb + before[u] + incl[u] - 1;
+        if (pos < a.out_cap) {
+          static_cast<PR*>(a.out_r)[pos] = (PR)t.r[m[u]].v;
+          static_cast<PS*>(a.out_s)[pos] = (PS)x[u].v;
+        }
+      }
+      return;
+    }
 #pragma unroll
     for (int u = 0; u < U; u++) {
       if (!c[u]) continue;
