@@ -15,6 +15,6 @@ NH=$((3*4)); NS=$((3*4)); NB=3
 if [ "$CFG" = "c1" ]; then NH=6; NS=6; fi
 for K in k_hist:$NH k_scatter:$NS k_build_probe:$NB; do
   N=${K%%:*}; S=${K##*:}
-  timeout 600 ncu --set full --clock-control none --import-source on -k regex:$N -s $S -c 2 -o gpurun_out/full_${TAG}_${CFG}_${N} $B > /dev/null 2>&1
+  timeout 600 ncu --set full --clock-control none --import-source on -k regex:$N -s $S -c 1 -o gpurun_out/full_${TAG}_${CFG}_${N} $B > /dev/null 2>&1
 done
 ls -la gpurun_out
