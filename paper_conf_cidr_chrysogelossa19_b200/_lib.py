@@ -80,7 +80,7 @@ class hape_plan(ctypes.Structure):
 def _load() -> ctypes.CDLL:
     if not os.path.exists(LIB_PATH):
         raise ImportError(f"{LIB_PATH} is missing: run __graft_entry__.build() "
-                          "(python -m paper_conf_cidr_chrysogelossa19_b200.build); there is no fallback")
+                          "(python __graft_entry__.py); there is no fallback")
     lib = ctypes.CDLL(LIB_PATH)
     P = ctypes.POINTER
     vp = ctypes.c_void_p

@@ -1,6 +1,6 @@
 """Build libhape.so in-tree with nvcc for sm_100a (no JIT cache, no torch ext).
 
-    python -m paper_conf_cidr_chrysogelossa19_b200.build
+    python __graft_entry__.py   (loads this file by path; the package import needs the library)
 """
 from __future__ import annotations
 
