@@ -247,8 +247,10 @@ static size_t tup_bytes(int kw, int pw) { return (kw + pw) <= 8 ? 8 : 16; }
 template <int KW, int PW, bool AOS>
 static void hist_t(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* hist, uint32_t* rowsum) {
   const unsigned grid = m.nseg * m.cps;
-  k_hist<KW, PW, AOS><<<grid, HIST_THREADS, (size_t)P * 4, h->stream>>>(s.in, m, bf, h->cfg.part_fn == HAPE_PART_IDENTITY,
-                                                                        P, hist, rowsum);
+  if (h->cfg.part_fn == HAPE_PART_IDENTITY)
+    k_hist<KW, PW, AOS, true><<<grid, HIST_THREADS, (size_t)P * 4, h->stream>>>(s.in, m, bf, P, hist, rowsum);
+  else
+    k_hist<KW, PW, AOS, false><<<grid, HIST_THREADS, (size_t)P * 4, h->stream>>>(s.in, m, bf, P, hist, rowsum);
 }
 
 static hape_status launch_hist(hape_join* h, int kw, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* hist,
@@ -278,45 +280,43 @@ static hape_status launch_scan(hape_join* h, SegMap m, uint32_t P, uint32_t* his
   return HAPE_OK;
 }
 
-template <int KW, int PW, bool AOS, class C>
+template <int KW, int PW, bool AOS, class C, bool IDENT>
 static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, const uint32_t* offs,
                              void* out) {
   const size_t smem = ScLayout<KW, PW, AOS, C>::bytes(P);
   static bool attr_set = false;
   if (!attr_set) {
-    CK(h, cudaFuncSetAttribute(k_scatter<KW, PW, AOS, C>, cudaFuncAttributeMaxDynamicSharedMemorySize, 220 * 1024));
+    CK(h, cudaFuncSetAttribute(k_scatter<KW, PW, AOS, C, IDENT>, cudaFuncAttributeMaxDynamicSharedMemorySize,
+                               220 * 1024));
     attr_set = true;
   }
   const unsigned grid = m.nseg * m.cps;
   if (grid == 0) return HAPE_OK;
-  k_scatter<KW, PW, AOS, C><<<grid, C::NT, smem, h->stream>>>(s.in, m, bf, h->cfg.part_fn == HAPE_PART_IDENTITY, P,
-                                                             offs, static_cast<Tup<KW, PW>*>(out));
+  k_scatter<KW, PW, AOS, C, IDENT><<<grid, C::NT, smem, h->stream>>>(s.in, m, bf, P, offs,
+                                                                   static_cast<Tup<KW, PW>*>(out));
   CK_LAUNCH(h);
   return HAPE_OK;
 }
 
-// scatter shape per tuple width; HAPE_SC selects alternatives (tuning only)
+// scatter shape per tuple width (measured best of the ScCfg sweep);
+// HAPE_SC=1 selects the destination-table variant (tuning only)
+template <int KW, int PW, bool AOS, bool IDENT>
+static hape_status scatter_i(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, const uint32_t* offs,
+                             void* out) {
+  static int v = [] { const char* e = getenv("HAPE_SC"); return e ? atoi(e) : 0; }();
+  if constexpr (KW + PW <= 8) {
+    if (v == 1) return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2, true>, IDENT>(h, s, m, bf, P, offs, out);
+    return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2>, IDENT>(h, s, m, bf, P, offs, out);
+  } else {
+    return scatter_t<KW, PW, AOS, ScCfg<256, 8, 2, 3>, IDENT>(h, s, m, bf, P, offs, out);
+  }
+}
+
 template <int KW, int PW, bool AOS>
 static hape_status scatter_v(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, const uint32_t* offs,
                              void* out) {
-  static int v = [] { const char* e = getenv("HAPE_SC"); return e ? atoi(e) : -1; }();
-  if constexpr (KW + PW <= 8) {
-    switch (v) {
-      case 1: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 2, 3>>(h, s, m, bf, P, offs, out);
-      case 2: return scatter_t<KW, PW, AOS, ScCfg<256, 16, 2, 3>>(h, s, m, bf, P, offs, out);
-      case 3: return scatter_t<KW, PW, AOS, ScCfg<256, 16, 3, 2>>(h, s, m, bf, P, offs, out);
-      case 4: return scatter_t<KW, PW, AOS, ScCfg<512, 16, 2, 1>>(h, s, m, bf, P, offs, out);
-      case 5: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 2, 2, true>>(h, s, m, bf, P, offs, out);
-      case 6: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2, true>>(h, s, m, bf, P, offs, out);
-      case 7: return scatter_t<KW, PW, AOS, ScCfg<256, 16, 2, 2, true>>(h, s, m, bf, P, offs, out);
-      default: return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2>>(h, s, m, bf, P, offs, out);
-    }
-  } else {
-    switch (v) {
-      case 1: return scatter_t<KW, PW, AOS, ScCfg<256, 8, 3, 2>>(h, s, m, bf, P, offs, out);
-      default: return scatter_t<KW, PW, AOS, ScCfg<256, 8, 2, 3>>(h, s, m, bf, P, offs, out);
-    }
-  }
+  if (h->cfg.part_fn == HAPE_PART_IDENTITY) return scatter_i<KW, PW, AOS, true>(h, s, m, bf, P, offs, out);
+  return scatter_i<KW, PW, AOS, false>(h, s, m, bf, P, offs, out);
 }
 
 static hape_status launch_scatter(hape_join* h, int kw, const Src& s, SegMap m, BitField bf, uint32_t P,

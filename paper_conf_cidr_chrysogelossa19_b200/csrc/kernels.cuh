@@ -50,10 +50,11 @@ __device__ __forceinline__ uint64_t fmix64(uint64_t x) {
 }
 
 // h(k): bijective mixer of the key bit pattern, or identity (P802-804)
-template <int KW>
-__device__ __forceinline__ uint64_t part_hash(typename UW<KW>::T k, int ident) {
-  if (ident) return (uint64_t)k;
-  if constexpr (KW == 4) return (uint64_t)fmix32(k);
+// (IDENT is a template parameter: the per-tuple paths carry no branch on it)
+template <int KW, bool IDENT>
+__device__ __forceinline__ uint64_t part_hash(typename UW<KW>::T k) {
+  if constexpr (IDENT) return (uint64_t)k;
+  else if constexpr (KW == 4) return (uint64_t)fmix32(k);
   else return fmix64(k);
 }
 
@@ -251,6 +252,13 @@ __device__ __forceinline__ void bulk_g2s(void* dst, const void* src, uint32_t by
       "l"(src), "r"(bytes), "r"(smem_u32(bar)), "l"(pol)
       : "memory");
 }
+// L2 prefetch of [src, src + bytes) rounded out to 16-byte boundaries (bulk
+// engine, no destination, no completion tracking)
+__device__ __forceinline__ void bulk_prefetch_l2(const void* src, size_t bytes) {
+  const uintptr_t a = reinterpret_cast<uintptr_t>(src);
+  const uintptr_t a0 = a & ~(uintptr_t)15, a1 = (a + bytes + 15) & ~(uintptr_t)15;
+  asm volatile("cp.async.bulk.prefetch.L2.global [%0], %1;" ::"l"(a0), "r"((uint32_t)(a1 - a0)) : "memory");
+}
 // copy [src, src + bytes) rounded out to 16-byte boundaries; returns the
 // byte offset of src inside the destination buffer
 __device__ __forceinline__ uint32_t bulk_g2s_any(void* dst, const void* src, size_t bytes, uint64_t* bar,
@@ -273,9 +281,9 @@ __device__ __forceinline__ uint32_t bulk_g2s_any(void* dst, const void* src, siz
 constexpr int HIST_THREADS = 512;
 constexpr int HIST_VEC = 4;
 
-template <int KW, int PW, bool AOS>
+template <int KW, int PW, bool AOS, bool IDENT>
 __global__ void __launch_bounds__(HIST_THREADS)
-k_hist(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, uint32_t* __restrict__ hist,
+k_hist(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ hist,
        uint32_t* __restrict__ rowsum) {
   extern __shared__ uint32_t sh_cnt[];
   using K = typename UW<KW>::T;
@@ -296,9 +304,9 @@ k_hist(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, uint32_t* __rest
   const uint32_t nvec = (hi - vlo) / PER;
   const uint32_t vhi = vlo + nvec * PER;
   for (uint32_t i = lo + threadIdx.x; i < vlo; i += HIST_THREADS)
-    atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(key_of(base[i]), ident), bf)], 1u);
+    atomicAdd(&sh_cnt[bucket_of(part_hash<KW, IDENT>(key_of(base[i])), bf)], 1u);
   for (uint32_t i = vhi + threadIdx.x; i < hi; i += HIST_THREADS)
-    atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(key_of(base[i]), ident), bf)], 1u);
+    atomicAdd(&sh_cnt[bucket_of(part_hash<KW, IDENT>(key_of(base[i])), bf)], 1u);
   const uint4* __restrict__ vk = reinterpret_cast<const uint4*>(base + vlo);
   uint32_t v = threadIdx.x;
   for (; v + (HIST_VEC - 1) * HIST_THREADS < nvec; v += HIST_VEC * HIST_THREADS) {
@@ -309,14 +317,14 @@ k_hist(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, uint32_t* __rest
     for (int u = 0; u < HIST_VEC; u++) {
       const E* ee = reinterpret_cast<const E*>(&w[u]);
 #pragma unroll
-      for (int e = 0; e < PER; e++) atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(key_of(ee[e]), ident), bf)], 1u);
+      for (int e = 0; e < PER; e++) atomicAdd(&sh_cnt[bucket_of(part_hash<KW, IDENT>(key_of(ee[e])), bf)], 1u);
     }
   }
   for (; v < nvec; v += HIST_THREADS) {
     const uint4 w = __ldcs(vk + v);
     const E* ee = reinterpret_cast<const E*>(&w);
 #pragma unroll
-    for (int e = 0; e < PER; e++) atomicAdd(&sh_cnt[bucket_of(part_hash<KW>(key_of(ee[e]), ident), bf)], 1u);
+    for (int e = 0; e < PER; e++) atomicAdd(&sh_cnt[bucket_of(part_hash<KW, IDENT>(key_of(ee[e])), bf)], 1u);
   }
   __syncthreads();
   const uint32_t row0 = seg * P;
@@ -442,9 +450,9 @@ __device__ __forceinline__ void sc_issue(const PartIn& in, uint32_t t0, uint32_t
   }
 }
 
-template <int KW, int PW, bool AOS, class C>
+template <int KW, int PW, bool AOS, class C, bool IDENT>
 __global__ void __launch_bounds__(C::NT, C::MINB)
-k_scatter(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, const uint32_t* __restrict__ offsets,
+k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, const uint32_t* __restrict__ offsets,
           Tup<KW, PW>* __restrict__ out) {
   using K = typename UW<KW>::T;
   using V = typename UW<PW>::T;
@@ -514,7 +522,7 @@ k_scatter(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, const uint32_
       for (int u = 0; u < ITEMS; u++) x[u] = load(u * NT + threadIdx.x);
 #pragma unroll
       for (int u = 0; u < ITEMS; u++) {
-        const uint32_t b = bucket_of(part_hash<KW>(x[u].k, ident), bf);
+        const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
         br[u] = (b << 16) | atomicAdd(&s_cnt[b], 1u);
       }
     } else {
@@ -523,7 +531,7 @@ k_scatter(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, const uint32_
         const uint32_t i = u * NT + threadIdx.x;
         if (i < tn) {
           x[u] = load(i);
-          const uint32_t b = bucket_of(part_hash<KW>(x[u].k, ident), bf);
+          const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
           br[u] = (b << 16) | atomicAdd(&s_cnt[b], 1u);
         }
       }
@@ -559,12 +567,20 @@ k_scatter(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, const uint32_
     __syncthreads();  // B: run starts known
     // phase 3: reorder the tile in shared memory (in place), bucket runs consecutive
     if (full) {
+      // all run-start loads first, then the stores: the compiler cannot tell
+      // s_tile from s_st apart, so interleaving them serialises on LDS latency
+      uint32_t pos[ITEMS];
 #pragma unroll
-      for (int u = 0; u < ITEMS; u++) {
-        const uint32_t pos = s_st[br[u] >> 16] + (br[u] & 0xFFFFu);
-        s_tile[pos] = x[u];
-        if constexpr (C::DST) s_dst[pos] = s_dl[br[u] >> 16] + pos;
+      for (int u = 0; u < ITEMS; u++) pos[u] = s_st[br[u] >> 16] + (br[u] & 0xFFFFu);
+      if constexpr (C::DST) {
+        uint32_t dl[ITEMS];
+#pragma unroll
+        for (int u = 0; u < ITEMS; u++) dl[u] = s_dl[br[u] >> 16];
+#pragma unroll
+        for (int u = 0; u < ITEMS; u++) s_dst[pos[u]] = dl[u] + pos[u];
       }
+#pragma unroll
+      for (int u = 0; u < ITEMS; u++) s_tile[pos[u]] = x[u];
     } else {
 #pragma unroll
       for (int u = 0; u < ITEMS; u++)
@@ -582,7 +598,7 @@ k_scatter(PartIn in, SegMap m, BitField bf, int ident, uint32_t P, const uint32_
     // random shared-memory store + load)
     auto dst_of = [&](uint32_t i, const Tp& y) -> uint32_t {
       if constexpr (C::DST) return s_dst[i];
-      else return s_dl[bucket_of(part_hash<KW>(y.k, ident), bf)] + i;
+      else return s_dl[bucket_of(part_hash<KW, IDENT>(y.k), bf)] + i;
     };
     if (full) {
 #pragma unroll
@@ -709,23 +725,26 @@ struct JnTable {
   bool dup;                 // the chunk holds some key twice (bag semantics path)
 };
 
-// Probe U S tuples per consumer thread: j = base + u*256 + tid.
-template <int KW, int PRW, int PSW, bool MAT, int U>
-__device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const JoinArgs& a, uint32_t base,
-                                               uint32_t s_hi, JnAcc& acc, uint32_t* s_wsum,
-                                               unsigned long long* s_wbase) {
-  using TS = Tup<KW, PSW>;
-  using PR = typename UW<PRW>::S;
-  using PS = typename UW<PSW>::S;
-  const TS* __restrict__ sT = static_cast<const TS*>(a.st);
-  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
-  TS x[U];
-  uint32_t e0[U];
+// Load U S tuples per consumer thread: j = base + u*256 + tid.
+template <int KW, int PSW, int U>
+__device__ __forceinline__ void jn_load_batch(const JoinArgs& a, uint32_t base, uint32_t s_hi, Tup<KW, PSW> (&x)[U]) {
+  const Tup<KW, PSW>* __restrict__ sT = static_cast<const Tup<KW, PSW>*>(a.st);
 #pragma unroll
   for (int u = 0; u < U; u++) {
     const uint32_t j = base + u * JN_CONSUMERS + threadIdx.x;
     if (j < s_hi) x[u] = ldcs_tup(sT + j);
   }
+}
+
+// Probe the U S tuples x[] (loaded by jn_load_batch for the same base).
+template <int KW, int PRW, int PSW, bool MAT, int U>
+__device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const JoinArgs& a, uint32_t base,
+                                               uint32_t s_hi, const Tup<KW, PSW> (&x)[U], JnAcc& acc,
+                                               uint32_t* s_wsum, unsigned long long* s_wbase) {
+  using PR = typename UW<PRW>::S;
+  using PS = typename UW<PSW>::S;
+  const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
+  uint32_t e0[U];
 #pragma unroll
   for (int u = 0; u < U; u++) {
     const uint32_t j = base + u * JN_CONSUMERS + threadIdx.x;
@@ -837,7 +856,6 @@ k_build_probe(JoinArgs a) {
   __shared__ uint32_t s_wsum[JN_CONSUMERS / 32];
   __shared__ unsigned long long s_wbase[JN_CONSUMERS / 32];
   __shared__ unsigned long long s_red[4][JN_THREADS / 32];
-  __shared__ uint32_t s_dup;
 
   const uint32_t nslots = 1u << a.slot_bits;
   const int lane = threadIdx.x & 31, warp = threadIdx.x >> 5;
@@ -855,6 +873,8 @@ k_build_probe(JoinArgs a) {
       const uint64_t pol = policy_evict_first();
       const uint32_t n_items = *a.n_items;
       const TR* rT = static_cast<const TR*>(a.rt);
+      using TS = Tup<KW, PSW>;
+      const TS* sT = static_cast<const TS*>(a.st);
       uint32_t stage = 0;
       for (uint32_t it = blockIdx.x; it < n_items; it += gridDim.x) {
         const uint2 item = a.items[it];
@@ -871,6 +891,8 @@ k_build_probe(JoinArgs a) {
           s_meta[bi] = JnStage{nr, (uint32_t)(ra - r0), s_lo, s_hi};
           mbar_expect_tx(&full[bi], (uint32_t)(r1 - r0));
           bulk_g2s(ring + bi * RB, reinterpret_cast<const void*>(r0), (uint32_t)(r1 - r0), &full[bi], pol);
+          // warm L2 with the stage's S slice: the consumers reach it a stage later
+          if (c_lo == r_lo && s_hi > s_lo) bulk_prefetch_l2(sT + s_lo, (size_t)(s_hi - s_lo) * sizeof(TS));
         }
       }
       const uint32_t bi = stage & 1, ph = (stage >> 1) & 1;
@@ -892,27 +914,43 @@ k_build_probe(JoinArgs a) {
       const TR* r = reinterpret_cast<const TR*>(ring + bi * RB + st.off);
       consumer_sync();
       // ---- build (a11): chained table via atomicExch on the heads
+      // the first S batch is loaded before the build so its latency hides
+      // behind the table construction
+      constexpr uint32_t BATCH = JN_U * JN_CONSUMERS;
+      Tup<KW, PSW> xs[JN_U];
+      if (st.s_lo + BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U>(a, st.s_lo, st.s_hi, xs);
       if (!(a.dbg & 4u))
         for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
           s_next[i] = (uint16_t)atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], i);
-      if (threadIdx.x == 0) s_dup = 0;
       consumer_sync();
-      // bag semantics walk every chain to its end; a caller-declared unique
-      // build side (HAPE_FLAG_R_UNIQUE, a primary key) stops at the first match
-      if (threadIdx.x == 0) s_dup = a.r_unique ? 0u : 1u;
-      consumer_sync();
-      // ---- probe (a12): stream the S slice
-      const JnTable<KW, PRW> tab{r, s_next, s_head, a.slot_bits, s_dup != 0};
+      // ---- probe (a12): stream the S slice.  Bag semantics walk every chain
+      // to its end; a caller-declared unique build side (HAPE_FLAG_R_UNIQUE, a
+      // primary key) stops at the first match.  Full batches are software
+      // pipelined: batch b+1 is loaded into registers while b is probed.
+      const JnTable<KW, PRW> tab{r, s_next, s_head, a.slot_bits, a.r_unique == 0};
       uint32_t base = st.s_lo;
-      for (; base + JN_U * JN_CONSUMERS <= st.s_hi; base += JN_U * JN_CONSUMERS)
-        jn_probe_batch<KW, PRW, PSW, MAT, JN_U>(tab, a, base, st.s_hi, acc, s_wsum, s_wbase);
+      while (base + BATCH <= st.s_hi) {
+        Tup<KW, PSW> x[JN_U];
+#pragma unroll
+        for (int u = 0; u < JN_U; u++) x[u] = xs[u];
+        if (base + 2 * BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U>(a, base + BATCH, st.s_hi, xs);
+        jn_probe_batch<KW, PRW, PSW, MAT, JN_U>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+        base += BATCH;
+      }
       const uint32_t rem = st.s_hi > base ? st.s_hi - base : 0;
-      if (rem > 2 * JN_CONSUMERS)
-        jn_probe_batch<KW, PRW, PSW, MAT, 4>(tab, a, base, st.s_hi, acc, s_wsum, s_wbase);
-      else if (rem > JN_CONSUMERS)
-        jn_probe_batch<KW, PRW, PSW, MAT, 2>(tab, a, base, st.s_hi, acc, s_wsum, s_wbase);
-      else if (rem > 0)
-        jn_probe_batch<KW, PRW, PSW, MAT, 1>(tab, a, base, st.s_hi, acc, s_wsum, s_wbase);
+      if (rem > 2 * JN_CONSUMERS) {
+        Tup<KW, PSW> x[4];
+        jn_load_batch<KW, PSW, 4>(a, base, st.s_hi, x);
+        jn_probe_batch<KW, PRW, PSW, MAT, 4>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+      } else if (rem > JN_CONSUMERS) {
+        Tup<KW, PSW> x[2];
+        jn_load_batch<KW, PSW, 2>(a, base, st.s_hi, x);
+        jn_probe_batch<KW, PRW, PSW, MAT, 2>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+      } else if (rem > 0) {
+        Tup<KW, PSW> x[1];
+        jn_load_batch<KW, PSW, 1>(a, base, st.s_hi, x);
+        jn_probe_batch<KW, PRW, PSW, MAT, 1>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+      }
       consumer_sync();  // everyone is done with heads/next and ring buffer bi
       if (threadIdx.x == 0) mbar_arrive(&empty[bi]);
     }

@@ -1,9 +1,12 @@
 #!/bin/bash
 # one GPU round-trip: parity tests, bench line, per-launch ncu list
+#   NO_TESTS=1 skips pytest, NO_NCU=1 skips the launch list, BENCH_ARGS passes through
 TAG=${1:-x}
 mkdir -p gpurun_out
-timeout 600 python -m pytest tests -m gpu -x -q 2>&1 | tail -5 > gpurun_out/tests_$TAG.log
+if [ -z "$NO_TESTS" ]; then
+timeout 900 python -m pytest tests -m gpu -x -q 2>&1 | tail -5 > gpurun_out/tests_$TAG.log
 cat gpurun_out/tests_$TAG.log
+fi
 timeout 300 python bench.py ${BENCH_ARGS} 2>&1 | tail -2 > gpurun_out/bench_$TAG.log
 cat gpurun_out/bench_$TAG.log
 if [ -z "$NO_NCU" ]; then
