@@ -720,6 +720,10 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
     static const uint32_t jn_dbg = [] { const char* e = getenv("HAPE_JN_DBG"); return e ? (uint32_t)atoi(e) : 0u; }();
     ja.dbg = jn_dbg;  // timing experiments only: results are wrong when set
     ja.r_unique = (c.flags & HAPE_FLAG_R_UNIQUE) ? 1u : 0u;
+    // L2 warm-up window per stage: the head of each S slice (a whole C2 slice;
+    // larger slices would thrash L2 a stage ahead of their use)
+    static const int pf_env = [] { const char* e = getenv("HAPE_JN_PF"); return e ? atoi(e) : -1; }();
+    ja.pf_bytes = pf_env >= 0 ? (uint32_t)pf_env : 32768u;
     CKS(launch_join(h, kw, prw, psw, ja, mat, &pl.join_ctas));
     mark(h, HAPE_STAGE_FINALIZE);
     // local result: acc[4], out_ctr, ctrs

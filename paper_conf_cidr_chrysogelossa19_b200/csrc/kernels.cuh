@@ -693,6 +693,7 @@ struct JoinArgs {
   void* out_r; void* out_s; unsigned long long out_cap; unsigned long long* out_ctr;
   uint32_t dbg;                              // timing experiments only (HAPE_JN_DBG); 0 in production
   uint32_t r_unique;                         // caller guarantees unique R keys (HAPE_FLAG_R_UNIQUE)
+  uint32_t pf_bytes;                         // L2 prefetch window at the head of each S slice (0 = off)
 };
 
 struct JnStage {
@@ -892,7 +893,8 @@ k_build_probe(JoinArgs a) {
           mbar_expect_tx(&full[bi], (uint32_t)(r1 - r0));
           bulk_g2s(ring + bi * RB, reinterpret_cast<const void*>(r0), (uint32_t)(r1 - r0), &full[bi], pol);
           // warm L2 with the stage's S slice: the consumers reach it a stage later
-          if (c_lo == r_lo && s_hi > s_lo) bulk_prefetch_l2(sT + s_lo, (size_t)(s_hi - s_lo) * sizeof(TS));
+          if (c_lo == r_lo && s_hi > s_lo && a.pf_bytes)
+            bulk_prefetch_l2(sT + s_lo, min((size_t)(s_hi - s_lo) * sizeof(TS), (size_t)a.pf_bytes));
         }
       }
       const uint32_t bi = stage & 1, ph = (stage >> 1) & 1;
@@ -917,8 +919,12 @@ k_build_probe(JoinArgs a) {
       // the first S batch is loaded before the build so its latency hides
       // behind the table construction
       constexpr uint32_t BATCH = JN_U * JN_CONSUMERS;
+      // (materialising kernels hold more live state: there the batch is
+      // loaded just before it is probed -- HAPE measured the pipelined form 2x
+      // slower for C3)
+      constexpr bool PIPE = !MAT;
       Tup<KW, PSW> xs[JN_U];
-      if (st.s_lo + BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U>(a, st.s_lo, st.s_hi, xs);
+      if (PIPE && st.s_lo + BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U>(a, st.s_lo, st.s_hi, xs);
       if (!(a.dbg & 4u))
         for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
           s_next[i] = (uint16_t)atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], i);
@@ -931,9 +937,13 @@ k_build_probe(JoinArgs a) {
       uint32_t base = st.s_lo;
       while (base + BATCH <= st.s_hi) {
         Tup<KW, PSW> x[JN_U];
+        if constexpr (PIPE) {
 #pragma unroll
-        for (int u = 0; u < JN_U; u++) x[u] = xs[u];
-        if (base + 2 * BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U>(a, base + BATCH, st.s_hi, xs);
+          for (int u = 0; u < JN_U; u++) x[u] = xs[u];
+          if (base + 2 * BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U>(a, base + BATCH, st.s_hi, xs);
+        } else {
+          jn_load_batch<KW, PSW, JN_U>(a, base, st.s_hi, x);
+        }
         jn_probe_batch<KW, PRW, PSW, MAT, JN_U>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
         base += BATCH;
       }
