@@ -278,11 +278,22 @@ def main():
         "build_probe": t * (nr_j + ns_j) + (2 * pw * res.n_written if materialize else 0),
         "devpart": (kw + 2 * t) * (nr_loc + ns_loc),
     }
-    if res.passes < 2:
-        alg.pop("hist2"); alg.pop("scatter2")
+    # two-pass plans with bits[0]+bits[1] <= 16 count both passes' buckets in
+    # the one read of the keys (k_hist_joint, stage hist1); k_joint_reduce
+    # (stage scan1, a few MB of per-SM partials) gives both passes' bounds and
+    # both scatters claim their runs: there is no pass-2 histogram read
+    joint = (res.passes == 2 and 6 <= res.bits[0] + res.bits[1] <= 16
+             and os.environ.get("HAPE_JOINT", "1") != "0")
     kernel_name = {"hist1": "k_hist pass 1 (R+S)", "scatter1": "k_scatter pass 1 (R+S)",
                    "hist2": "k_hist pass 2 (R+S)", "scatter2": "k_scatter pass 2 (R+S)",
                    "build_probe": "k_build_probe", "devpart": "device partition (hist+scan+scatter)"}
+    if joint:
+        alg.pop("hist2")
+        kernel_name["hist1"] = "k_hist_joint (pass-1 and pass-2 buckets, R+S)"
+        kernel_name["scatter1"] = "k_scatter pass 1, claiming (R+S)"
+        kernel_name["scatter2"] = "k_scatter pass 2, claiming (R+S)"
+    if res.passes < 2:
+        alg.pop("hist2", None); alg.pop("scatter2")
     dom = max((k for k in alg if stage_avg.get(k, 0) > 0), key=lambda k: stage_avg[k])
     peak, peak_src = load_peaks()
     per_stage = {}

@@ -270,6 +270,72 @@ static hape_status launch_hist(hape_join* h, int kw, const Src& s, SegMap m, Bit
   return HAPE_OK;
 }
 
+// Two-pass plans with B1 + B2 <= 16 count both passes' buckets in one read of
+// the keys (k_hist_joint) and run pass 2 as a claiming scatter.  HAPE_JOINT=0
+// forces the separate pass-2 histogram (tests compare both forms).
+static bool use_joint(const hape_plan& pl) {
+  static const int env = [] { const char* e = getenv("HAPE_JOINT"); return e ? atoi(e) : 1; }();
+  return env != 0 && pl.passes == 2 && pl.bits[0] + pl.bits[1] <= 16 && pl.bits[0] + pl.bits[1] >= 6 &&
+         pl.bits[1] >= 1;
+}
+
+static uint32_t joint_grid(const hape_join* h, uint32_t nchunks) {
+  return std::max<uint32_t>(1, std::min<uint32_t>((uint32_t)h->num_sms, nchunks));
+}
+
+static size_t joint_smem(uint32_t P1, uint32_t P2) { return (size_t)P1 * P2 * 2 + (size_t)P1 * 4; }
+
+template <int KW, int PW, bool AOS, bool IDENT>
+static hape_status hist_joint_t(hape_join* h, const Src& s, SegMap m, BitField bf1, BitField bf2, uint32_t P1,
+                                uint32_t P2, uint32_t* rowsum, uint16_t* part, uint32_t* ovf) {
+  auto kern = k_hist_joint<KW, PW, AOS, IDENT>;
+  static bool attr_set = false;
+  if (!attr_set) {
+    CK(h, cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024));
+    attr_set = true;
+  }
+  const uint32_t nch = m.nseg * m.cps;
+  kern<<<joint_grid(h, nch), HJ_THREADS, joint_smem(P1, P2), h->stream>>>(s.in, m, bf1, bf2, P1, P2, rowsum, part,
+                                                                        ovf);
+  return HAPE_OK;
+}
+
+template <int KW, int PW, bool AOS>
+static hape_status hist_joint_i(hape_join* h, const Src& s, SegMap m, BitField bf1, BitField bf2, uint32_t P1,
+                                uint32_t P2, uint32_t* rowsum, uint16_t* part, uint32_t* ovf) {
+  if (h->cfg.part_fn == HAPE_PART_IDENTITY)
+    return hist_joint_t<KW, PW, AOS, true>(h, s, m, bf1, bf2, P1, P2, rowsum, part, ovf);
+  return hist_joint_t<KW, PW, AOS, false>(h, s, m, bf1, bf2, P1, P2, rowsum, part, ovf);
+}
+
+static hape_status launch_hist_joint(hape_join* h, int kw, const Src& s, SegMap m, BitField bf1, BitField bf2,
+                                     uint32_t P1, uint32_t P2, uint32_t* rowsum, uint16_t* part, uint32_t* ovf) {
+  if (m.nseg * m.cps == 0) return HAPE_OK;
+  const int pw = s.pw;
+  hape_status st;
+  if (s.aos) {
+    if (kw == 4 && pw == 4) st = hist_joint_i<4, 4, true>(h, s, m, bf1, bf2, P1, P2, rowsum, part, ovf);
+    else if (kw == 4) st = hist_joint_i<4, 8, true>(h, s, m, bf1, bf2, P1, P2, rowsum, part, ovf);
+    else if (pw == 4) st = hist_joint_i<8, 4, true>(h, s, m, bf1, bf2, P1, P2, rowsum, part, ovf);
+    else st = hist_joint_i<8, 8, true>(h, s, m, bf1, bf2, P1, P2, rowsum, part, ovf);
+  } else {
+    if (kw == 4) st = hist_joint_i<4, 4, false>(h, s, m, bf1, bf2, P1, P2, rowsum, part, ovf);
+    else st = hist_joint_i<8, 8, false>(h, s, m, bf1, bf2, P1, P2, rowsum, part, ovf);
+  }
+  CKS(st);
+  CK_LAUNCH(h);
+  return HAPE_OK;
+}
+
+static hape_status launch_joint_reduce(hape_join* h, const uint16_t* part, uint32_t nparts, const uint32_t* ovf,
+                                       const uint32_t* rowsum, uint32_t P1, uint32_t P2, uint32_t* bounds1,
+                                       uint32_t* cursor1, uint32_t* bounds2, uint32_t* cursor2) {
+  k_joint_reduce<<<P1, JR_THREADS, 0, h->stream>>>(part, nparts, ovf, rowsum, P1, P2, bounds1, cursor1, bounds2,
+                                                   cursor2);
+  CK_LAUNCH(h);
+  return HAPE_OK;
+}
+
 static hape_status launch_scan(hape_join* h, SegMap m, uint32_t P, uint32_t* hist, const uint32_t* rowsum,
                                uint32_t* bounds_out) {
   uint32_t rpc = std::max<uint32_t>(1, SCAN_TILE / m.cps);
@@ -280,19 +346,19 @@ static hape_status launch_scan(hape_join* h, SegMap m, uint32_t P, uint32_t* his
   return HAPE_OK;
 }
 
-template <int KW, int PW, bool AOS, class C, bool IDENT>
-static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, const uint32_t* offs,
+template <int KW, int PW, bool AOS, class C, bool IDENT, bool CLAIM>
+static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* offs,
                              void* out) {
   const size_t smem = ScLayout<KW, PW, AOS, C>::bytes(P);
   static bool attr_set = false;
   if (!attr_set) {
-    CK(h, cudaFuncSetAttribute(k_scatter<KW, PW, AOS, C, IDENT>, cudaFuncAttributeMaxDynamicSharedMemorySize,
+    CK(h, cudaFuncSetAttribute(k_scatter<KW, PW, AOS, C, IDENT, CLAIM>, cudaFuncAttributeMaxDynamicSharedMemorySize,
                                220 * 1024));
     attr_set = true;
   }
   const unsigned grid = m.nseg * m.cps;
   if (grid == 0) return HAPE_OK;
-  k_scatter<KW, PW, AOS, C, IDENT><<<grid, C::NT, smem, h->stream>>>(s.in, m, bf, P, offs,
+  k_scatter<KW, PW, AOS, C, IDENT, CLAIM><<<grid, C::NT, smem, h->stream>>>(s.in, m, bf, P, offs,
                                                                    static_cast<Tup<KW, PW>*>(out));
   CK_LAUNCH(h);
   return HAPE_OK;
@@ -300,33 +366,37 @@ static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, 
 
 // scatter shape per tuple width (measured best of the ScCfg sweep);
 // HAPE_SC=1 selects the destination-table variant (tuning only)
-template <int KW, int PW, bool AOS, bool IDENT>
-static hape_status scatter_i(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, const uint32_t* offs,
+template <int KW, int PW, bool AOS, bool IDENT, bool CLAIM>
+static hape_status scatter_i(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* offs,
                              void* out) {
   static int v = [] { const char* e = getenv("HAPE_SC"); return e ? atoi(e) : 0; }();
   if constexpr (KW + PW <= 8) {
-    if (v == 1) return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2, true>, IDENT>(h, s, m, bf, P, offs, out);
-    return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2>, IDENT>(h, s, m, bf, P, offs, out);
+    if (v == 1) return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2, true>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
+    return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
   } else {
-    return scatter_t<KW, PW, AOS, ScCfg<256, 8, 2, 3>, IDENT>(h, s, m, bf, P, offs, out);
+    return scatter_t<KW, PW, AOS, ScCfg<256, 8, 2, 3>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
   }
 }
 
 template <int KW, int PW, bool AOS>
-static hape_status scatter_v(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, const uint32_t* offs,
-                             void* out) {
-  if (h->cfg.part_fn == HAPE_PART_IDENTITY) return scatter_i<KW, PW, AOS, true>(h, s, m, bf, P, offs, out);
-  return scatter_i<KW, PW, AOS, false>(h, s, m, bf, P, offs, out);
+static hape_status scatter_v(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* offs,
+                             void* out, bool claim) {
+  if (claim) {
+    if (h->cfg.part_fn == HAPE_PART_IDENTITY) return scatter_i<KW, PW, AOS, true, true>(h, s, m, bf, P, offs, out);
+    return scatter_i<KW, PW, AOS, false, true>(h, s, m, bf, P, offs, out);
+  }
+  if (h->cfg.part_fn == HAPE_PART_IDENTITY) return scatter_i<KW, PW, AOS, true, false>(h, s, m, bf, P, offs, out);
+  return scatter_i<KW, PW, AOS, false, false>(h, s, m, bf, P, offs, out);
 }
 
 static hape_status launch_scatter(hape_join* h, int kw, const Src& s, SegMap m, BitField bf, uint32_t P,
-                                  const uint32_t* offs, void* out) {
+                                  uint32_t* offs, void* out, bool claim = false) {
   const int pw = s.pw;
-#define HAPE_SC_DISPATCH(AOS)                                                 \
-  if (kw == 4 && pw == 4) return scatter_v<4, 4, AOS>(h, s, m, bf, P, offs, out); \
-  if (kw == 4) return scatter_v<4, 8, AOS>(h, s, m, bf, P, offs, out);            \
-  if (pw == 4) return scatter_v<8, 4, AOS>(h, s, m, bf, P, offs, out);            \
-  return scatter_v<8, 8, AOS>(h, s, m, bf, P, offs, out);
+#define HAPE_SC_DISPATCH(AOS)                                                        \
+  if (kw == 4 && pw == 4) return scatter_v<4, 4, AOS>(h, s, m, bf, P, offs, out, claim); \
+  if (kw == 4) return scatter_v<4, 8, AOS>(h, s, m, bf, P, offs, out, claim);            \
+  if (pw == 4) return scatter_v<8, 4, AOS>(h, s, m, bf, P, offs, out, claim);            \
+  return scatter_v<8, 8, AOS>(h, s, m, bf, P, offs, out, claim);
   if (s.aos) { HAPE_SC_DISPATCH(true) } else { HAPE_SC_DISPATCH(false) }
 #undef HAPE_SC_DISPATCH
 }
@@ -391,6 +461,10 @@ struct Carve {
 struct SideLayout {            // per relation
   uint32_t cps1 = 0, cps2 = 0;
   size_t hist1 = 0, rowsum1 = 0, bounds1 = 0, hist2 = 0, rowsum2 = 0, bounds2 = 0;
+  // joint path: hist2 holds the claim cursors [Q], rowsum2 the spill counts
+  // [Q] (zeroed), part the per-CTA 16-bit joint histograms [nparts][Q]
+  size_t part = 0;
+  uint32_t nparts = 0;
 };
 
 struct CallLayout {
@@ -420,9 +494,15 @@ static CallLayout layout_for(const hape_join* h, const hape_plan& pl, uint64_t n
   for (int s = 0; s < 2; s++) {
     SideLayout& S = L.side[s];
     S.cps1 = cps_for(h, ns[s], 1);
-    S.hist1 = cv.take(P1 * S.cps1 * 4);
+    S.hist1 = cv.take(P1 * (use_joint(pl) ? 1 : S.cps1) * 4);  // joint path: pass-1 claim cursors
     S.bounds1 = cv.take((P1 + 1) * 4);
-    if (pl.passes == 2) {
+    if (pl.passes == 2 && use_joint(pl)) {
+      S.cps2 = cps_for(h, ns[s], (uint32_t)P1);
+      S.hist2 = cv.take(Q * 4);
+      S.bounds2 = cv.take((Q + 1) * 4);
+      S.nparts = joint_grid(h, S.cps1);
+      S.part = cv.take((size_t)S.nparts * Q * 2);
+    } else if (pl.passes == 2) {
       S.cps2 = cps_for(h, ns[s], (uint32_t)P1);
       S.hist2 = cv.take(Q * S.cps2 * 4);
       S.bounds2 = cv.take((Q + 1) * 4);
@@ -464,25 +544,41 @@ static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const
     if (pl.passes == 2) m2[s] = SegMap{at<uint32_t>(h, L.side[s].bounds1), P1, L.side[s].cps2, io[s].in.n};
     s2[s] = Src{PartIn{nullptr, nullptr, io[s].p1}, true, io[s].in.n, io[s].in.pw};
   }
+  // joint path (use_joint): hist1 = k_hist_joint (both passes' buckets),
+  // scan1 = k_joint_reduce (bounds + claim cursors of both passes), both
+  // scatters claim; hist2 / scan2 are empty.  Workspace reuse: hist1 / hist2
+  // hold the pass-1 / pass-2 cursors, rowsum1 the row totals, rowsum2 the
+  // spilled counts (both zeroed per call).
+  const bool joint = use_joint(pl);
   auto hist1 = [&](int s) {
+    if (joint)
+      return launch_hist_joint(h, kw, io[s].in, m1[s], bf1, bf2, P1, P2, at<uint32_t>(h, L.side[s].rowsum1),
+                               at<uint16_t>(h, L.side[s].part), at<uint32_t>(h, L.side[s].rowsum2));
     return launch_hist(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1));
   };
   auto scan1 = [&](int s) {
+    if (joint)
+      return launch_joint_reduce(h, at<uint16_t>(h, L.side[s].part), L.side[s].nparts,
+                                 at<uint32_t>(h, L.side[s].rowsum2), at<uint32_t>(h, L.side[s].rowsum1), P1, P2,
+                                 at<uint32_t>(h, L.side[s].bounds1), at<uint32_t>(h, L.side[s].hist1),
+                                 at<uint32_t>(h, L.side[s].bounds2), at<uint32_t>(h, L.side[s].hist2));
     return launch_scan(h, m1[s], P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1),
                        at<uint32_t>(h, L.side[s].bounds1));
   };
   auto scatter1 = [&](int s) {
-    return launch_scatter(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), io[s].p1);
+    return launch_scatter(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), io[s].p1, joint);
   };
   auto hist2 = [&](int s) {
+    if (joint) return HAPE_OK;
     return launch_hist(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), at<uint32_t>(h, L.side[s].rowsum2));
   };
   auto scan2 = [&](int s) {
+    if (joint) return HAPE_OK;
     return launch_scan(h, m2[s], P2, at<uint32_t>(h, L.side[s].hist2), at<uint32_t>(h, L.side[s].rowsum2),
                        at<uint32_t>(h, L.side[s].bounds2));
   };
   auto scatter2 = [&](int s) {
-    return launch_scatter(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), io[s].p2);
+    return launch_scatter(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), io[s].p2, joint);
   };
   if (side1_ready) {
     for (int s = 0; s < nside; s++) {

@@ -336,6 +336,168 @@ k_hist(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ hist
 }
 
 // --------------------------------------------------------------------------
+// a6 for both passes in one read of the keys (two-pass plans with
+// B1 + B2 <= 16).  The pass-2 histogram is what the paper's "extra scan"
+// (P593-597) would re-read from the pass-1 output; here each key's pass-1 and
+// pass-2 buckets are counted together, as one JOINT bucket q = b1*P2 + b2:
+// a persistent CTA per SM walks chunks (blockIdx.x, +gridDim.x, ...) and
+// accumulates 16-bit shared-memory counters, two per 32-bit word (2^16 bins =
+// 128 KB).  Wrap-around is handled exactly from the atomic's return value:
+//   * the low half of word w counts bin 2w, the high half bin 2w+1;
+//   * an increment that finds its half at 0xFFFF wraps it: it adds 65536 to
+//     ovf[q] (u32, global);
+//   * a wrapping low half also carries 1 into the high half: ovf[q+1] -= 1,
+//     and if that carry wrapped the high half too (old word 0xFFFFFFFF),
+//     ovf[q+1] += 65536.
+// Each wrap is seen by exactly the atomic that causes it, so for every bin
+// count = half + ovf (mod 2^32), with no periodic checks.  Row totals go to
+// rowsum[b1] (the ovf deltas too), the counters to part[blockIdx.x][Q]
+// (coalesced, no atomics); k_joint_reduce turns the partials into both
+// passes' bounds and cursors, and both scatters claim their runs (k_scatter
+// CLAIM): no per-chunk histograms, no scan over them, one shared-memory
+// atomic per key.
+// --------------------------------------------------------------------------
+constexpr int HJ_THREADS = 1024;
+
+template <int KW, int PW, bool AOS, bool IDENT>
+__global__ void __launch_bounds__(HJ_THREADS, 1)
+k_hist_joint(PartIn in, SegMap m, BitField bf1, BitField bf2, uint32_t P1, uint32_t P2,
+             uint32_t* __restrict__ rowsum, uint16_t* __restrict__ part, uint32_t* __restrict__ ovf) {
+  extern __shared__ __align__(16) uint32_t sh_hj[];
+  using K = typename UW<KW>::T;
+  using E = typename std::conditional<AOS, Tup<KW, PW>, K>::type;
+  constexpr int ES = sizeof(E);
+  constexpr int PER = 16 / ES;
+  const uint32_t Q = P1 * P2, QW = Q / 2, WPR = P2 / 2;  // words (2 bins) per row
+  uint32_t* j16 = sh_hj;                // [QW] pairs of 16-bit counters, row-major
+  uint32_t* rowtot = j16 + QW;          // [P1] row totals
+  const E* __restrict__ base = static_cast<const E*>(AOS ? in.t : in.k);
+  auto key_of = [](const E& e) -> K {
+    if constexpr (AOS) return e.k;
+    else return e;
+  };
+  for (uint32_t i = threadIdx.x; i < QW; i += HJ_THREADS) j16[i] = 0;
+  for (uint32_t p = threadIdx.x; p < P1; p += HJ_THREADS) rowtot[p] = 0;
+  __syncthreads();
+  auto count = [&](K k) {
+    const uint64_t h = part_hash<KW, IDENT>(k);
+    const uint32_t q = bucket_of(h, bf1) * P2 + bucket_of(h, bf2);
+    const uint32_t sh = (q & 1u) * 16;
+    const uint32_t old = atomicAdd(&j16[q >> 1], 1u << sh);
+    if (((old >> sh) & 0xFFFFu) == 0xFFFFu) {  // this increment wrapped its half
+      const uint32_t p = q / P2;
+      atomicAdd(&ovf[q], 65536u);
+      uint32_t dr = 65536u;
+      if (!(q & 1u)) {  // the carry went into the neighbour's half
+        const uint32_t d = (old >> 16) == 0xFFFFu ? 65535u : 0xFFFFFFFFu;
+        atomicAdd(&ovf[q + 1], d);
+        dr += d;
+      }
+      atomicAdd(&rowsum[p], dr);
+    }
+  };
+  const uint32_t nchunks = m.nseg * m.cps;
+  for (uint32_t c = blockIdx.x; c < nchunks; c += gridDim.x) {
+    uint32_t seg, j, lo, hi;
+    seg_chunk(m, c, seg, j, lo, hi);
+    uint32_t vlo = lo;
+    while (vlo < hi && (reinterpret_cast<uintptr_t>(base + vlo) & 15)) vlo++;
+    const uint32_t nvec = (hi - vlo) / PER;
+    const uint32_t vhi = vlo + nvec * PER;
+    for (uint32_t i = lo + threadIdx.x; i < vlo; i += HJ_THREADS) count(key_of(base[i]));
+    for (uint32_t i = vhi + threadIdx.x; i < hi; i += HJ_THREADS) count(key_of(base[i]));
+    const uint4* __restrict__ vk = reinterpret_cast<const uint4*>(base + vlo);
+    uint32_t v = threadIdx.x;
+    for (; v + (HIST_VEC - 1) * HJ_THREADS < nvec; v += HIST_VEC * HJ_THREADS) {
+      uint4 w[HIST_VEC];
+#pragma unroll
+      for (int u = 0; u < HIST_VEC; u++) w[u] = __ldcs(vk + v + u * HJ_THREADS);
+#pragma unroll
+      for (int u = 0; u < HIST_VEC; u++) {
+        const E* ee = reinterpret_cast<const E*>(&w[u]);
+#pragma unroll
+        for (int e = 0; e < PER; e++) count(key_of(ee[e]));
+      }
+    }
+    for (; v < nvec; v += HJ_THREADS) {
+      const uint4 w = __ldcs(vk + v);
+      const E* ee = reinterpret_cast<const E*>(&w);
+#pragma unroll
+      for (int e = 0; e < PER; e++) count(key_of(ee[e]));
+    }
+  }
+  __syncthreads();
+  // row totals of the 16-bit counters: a warp covers 32 consecutive words;
+  // the lanes of one row differ only in the low log2(min(WPR, 32)) bits
+  // (QW is a multiple of 32: Q >= 64)
+  const uint32_t rseg = WPR < 32 ? WPR : 32u;
+  for (uint32_t w = threadIdx.x; w < QW; w += HJ_THREADS) {
+    const uint32_t x = j16[w];
+    uint32_t t = (x & 0xFFFFu) + (x >> 16);
+    for (uint32_t o = 1; o < rseg; o <<= 1) t += __shfl_xor_sync(0xffffffffu, t, o);
+    if (((threadIdx.x & 31) & (rseg - 1)) == 0) atomicAdd(&rowtot[w / WPR], t);
+  }
+  __syncthreads();
+  for (uint32_t p = threadIdx.x; p < P1; p += HJ_THREADS)
+    if (rowtot[p]) atomicAdd(&rowsum[p], rowtot[p]);
+  uint4* __restrict__ dst = reinterpret_cast<uint4*>(part + (size_t)blockIdx.x * Q);
+  const uint4* src = reinterpret_cast<const uint4*>(j16);
+  for (uint32_t i = threadIdx.x; i < QW / 4; i += HJ_THREADS) dst[i] = src[i];
+}
+
+// Row b1 = blockIdx.x: pass-1 bound = sum of the earlier rows' totals; sum
+// the per-CTA joint partials of the row (+ spills), scan its P2 counts and
+// emit the pass-2 sub-partition bounds; cursors (claim start points) for
+// both passes.  P2/2 words per row; thread groups split the partial index.
+constexpr int JR_THREADS = 512;
+
+__global__ void __launch_bounds__(JR_THREADS)
+k_joint_reduce(const uint16_t* __restrict__ part, uint32_t nparts, const uint32_t* __restrict__ ovf,
+               const uint32_t* __restrict__ rowsum, uint32_t P1, uint32_t P2, uint32_t* __restrict__ bounds1,
+               uint32_t* __restrict__ cursor1, uint32_t* __restrict__ bounds2, uint32_t* __restrict__ cursor2) {
+  __shared__ uint32_t row[4096];
+  __shared__ uint32_t wtmp[33];
+  __shared__ uint32_t s_b0;
+  const uint32_t Q = P1 * P2, p = blockIdx.x, WPR = P2 / 2;
+  // pass-1 bound of row p
+  uint32_t pre = 0;
+  for (uint32_t i = threadIdx.x; i < p; i += JR_THREADS) pre += rowsum[i];
+  for (int o = 16; o > 0; o >>= 1) pre += __shfl_xor_sync(0xffffffffu, pre, o);
+  if (threadIdx.x == 0) s_b0 = 0;
+  for (uint32_t b = threadIdx.x; b < P2; b += JR_THREADS) row[b] = ovf[p * P2 + b];
+  __syncthreads();
+  if ((threadIdx.x & 31) == 0 && pre) atomicAdd(&s_b0, pre);
+  // partial sums: thread (g0, w) adds words w of partials g0, g0+NG, ...
+  const uint32_t NG = WPR >= JR_THREADS ? 1u : JR_THREADS / WPR;
+  const uint32_t* pw = reinterpret_cast<const uint32_t*>(part);
+  for (uint32_t t = threadIdx.x; t < NG * WPR; t += JR_THREADS) {
+    const uint32_t w = t % WPR, g0 = t / WPR;
+    uint32_t lo = 0, hi = 0;
+#pragma unroll 4
+    for (uint32_t g = g0; g < nparts; g += NG) {
+      const uint32_t x = __ldg(pw + (size_t)g * (Q / 2) + p * WPR + w);
+      lo += x & 0xFFFFu;
+      hi += x >> 16;
+    }
+    atomicAdd(&row[2 * w], lo);
+    atomicAdd(&row[2 * w + 1], hi);
+  }
+  __syncthreads();
+  block_exscan_smem<JR_THREADS>(row, (int)P2, wtmp);
+  const uint32_t b0 = s_b0;
+  if (threadIdx.x == 0) { bounds1[p] = b0; cursor1[p] = b0; }
+  for (uint32_t b = threadIdx.x; b < P2; b += JR_THREADS) {
+    bounds2[p * P2 + b] = b0 + row[b];
+    cursor2[p * P2 + b] = b0 + row[b];
+  }
+  if (p == P1 - 1 && threadIdx.x == 0) {
+    const uint32_t n = b0 + rowsum[p];
+    bounds1[P1] = n;
+    bounds2[Q] = n;
+  }
+}
+
+// --------------------------------------------------------------------------
 // a7: exclusive prefix sum of the histograms -> absolute write offsets (in
 // place) and the partition bounds of the pass.  CTA (seg, row-group) scans a
 // contiguous tile of rows; the tile's base is the segment start plus the sum
@@ -450,9 +612,15 @@ __device__ __forceinline__ void sc_issue(const PartIn& in, uint32_t t0, uint32_t
   }
 }
 
-template <int KW, int PW, bool AOS, class C, bool IDENT>
+// CLAIM (pass 2 after k_hist_joint): `offsets` is the per-sub-partition
+// cursor array [seg*P + b]; each tile claims its bucket runs with one global
+// atomic per non-empty bucket instead of reading per-CTA offsets.  Runs of a
+// sub-partition then land in claim order (any order is a valid partition,
+// DESIGN.md R9); the claimed regions of concurrently running tiles are
+// adjacent, so L2 still merges the partial sectors at their seams.
+template <int KW, int PW, bool AOS, class C, bool IDENT, bool CLAIM = false>
 __global__ void __launch_bounds__(C::NT, C::MINB)
-k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, const uint32_t* __restrict__ offsets,
+k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ offsets,
           Tup<KW, PW>* __restrict__ out) {
   using K = typename UW<KW>::T;
   using V = typename UW<PW>::T;
@@ -472,7 +640,7 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, const uint32_t* __restri
 
   uint32_t seg, j, lo, hi;
   seg_chunk(m, blockIdx.x, seg, j, lo, hi);
-  const bool backward = (j & 1u) != 0;
+  const bool backward = !CLAIM && (j & 1u) != 0;
   const uint32_t row0 = seg * P;
   const size_t nflat = (size_t)m.nseg * P * m.cps;
   const uint32_t ntiles = (hi - lo + T - 1) / T;
@@ -487,8 +655,10 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, const uint32_t* __restri
     }
   }
   for (uint32_t p = threadIdx.x; p < P; p += NT) {
-    const size_t f = (size_t)(row0 + p) * m.cps + j;
-    s_cur[p] = backward ? (f + 1 < nflat ? offsets[f + 1] : m.n) : offsets[f];
+    if constexpr (!CLAIM) {
+      const size_t f = (size_t)(row0 + p) * m.cps + j;
+      s_cur[p] = backward ? (f + 1 < nflat ? offsets[f + 1] : m.n) : offsets[f];
+    }
     s_cnt[p] = 0;
   }
   __syncthreads();
@@ -549,17 +719,28 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, const uint32_t* __restri
       const uint32_t b0 = min(threadIdx.x * per, P), b1 = min(b0 + per, P);
       uint32_t sum = 0;
       for (uint32_t b = b0; b < b1; b++) sum += s_cnt[b];
+      // CLAIM with one bucket per thread: issue the claim now so its latency
+      // overlaps the scan and barrier X
+      uint32_t claim0 = 0;
+      if constexpr (CLAIM)
+        if (b1 == b0 + 1 && sum) claim0 = atomicAdd(&offsets[row0 + b0], sum);
       const uint32_t inc = warp_incl_scan(sum);
       if (lane == 31) s_wt[warp] = inc;
       __syncthreads();  // X
       uint32_t ex = inc - sum;
       for (int w = 0; w < warp; w++) ex += s_wt[w];
       for (uint32_t b = b0; b < b1; b++) {
-        const uint32_t c = s_cnt[b], cur = s_cur[b];
-        const uint32_t run = backward ? cur - c : cur;
+        const uint32_t c = s_cnt[b];
+        uint32_t run;
+        if constexpr (CLAIM) {
+          run = b1 == b0 + 1 ? claim0 : (c ? atomicAdd(&offsets[row0 + b], c) : 0u);
+        } else {
+          const uint32_t cur = s_cur[b];
+          run = backward ? cur - c : cur;
+          s_cur[b] = backward ? cur - c : cur + c;
+        }
         s_st[b] = ex;
         s_dl[b] = run - ex;
-        s_cur[b] = backward ? cur - c : cur + c;
         s_cnt[b] = 0;
         ex += c;
       }

@@ -317,3 +317,66 @@ def test_zipf_skew_vs_oracle(theta):
     check(res, want)
     if theta == 1.0:
         assert res.n_items > res.n_partitions  # the hot co-partitions were split into S slices
+
+
+# ---- the joint pass-1/pass-2 histogram (k_hist_joint) and the claiming pass 2
+def test_joint_histogram_row_spill_partitions():
+    # 2^24 tuples, 3/4 of them one key: every SM's 16-bit counters for that
+    # key's row would pass 65535, so the row-spill path runs; the partition
+    # invariants (bounds = bincount of the partition function, permutation)
+    # must still hold exactly
+    n = 1 << 24
+    rng = np.random.default_rng(5)
+    keys = rng.integers(-2**31, 2**31, n, dtype=np.int64).astype(np.int32)
+    keys[rng.random(n) < 0.75] = 12345
+    pays = np.arange(n, dtype=np.int32)
+    j = joiner(torch.int32, radix_passes=2, radix_bits=(8, 8))
+    ok, op, ob, plan = j.debug_partition(cuda(keys), cuda(pays))
+    ok, op, ob = ok.cpu().numpy(), op.cpu().numpy(), ob.cpu().numpy()
+    pid = partition.partition_id(keys, 8, 8)
+    assert np.array_equal(np.diff(ob), np.bincount(pid, minlength=1 << 16))
+    assert np.array_equal(np.sort(op), pays)
+    assert np.array_equal(ok, keys[op.astype(np.int64)])
+    assert np.array_equal(partition.partition_id(ok, 8, 8), np.repeat(np.arange(1 << 16), np.diff(ob)))
+
+
+def test_joint_histogram_skewed_join_vs_oracle():
+    # the same skew through the join (one S tuple of the hot key: count = its
+    # R multiplicity, the R co-partition is joined in chunks)
+    n = 1 << 22
+    rng = np.random.default_rng(6)
+    rk = rng.integers(-2**31, 2**31, n, dtype=np.int64).astype(np.int32)
+    rk[rng.random(n) < 0.6] = -7
+    rp = rng.integers(-2**31, 2**31, n, dtype=np.int64).astype(np.int32)
+    head = rk[:100000]
+    sk = np.concatenate([head[head != -7], np.array([-7], np.int32)])
+    sp = rng.integers(-2**31, 2**31, len(sk), dtype=np.int64).astype(np.int32)
+    want = oracle_res(rk, rp, sk, sp)
+    res = joiner(torch.int32, radix_passes=2, radix_bits=(8, 8)).join(cuda(rk), cuda(rp), cuda(sk), cuda(sp))
+    check(res, want)
+
+
+def test_separate_pass2_histogram_path_vs_oracle():
+    # HAPE_JOINT=0 forces the separate pass-2 histogram + offset scatter (the
+    # path plans with bits[0]+bits[1] > 16 take); read once per process, so it
+    # runs in a child process
+    import subprocess
+    import sys
+    import os
+    code = r'''
+import numpy as np, torch, datagen, oracle
+from paper_conf_cidr_chrysogelossa19_b200 import RadixJoin
+for cfg, nr, ns, kdt in (("c2", 1 << 20, (1 << 20) + 333, torch.int32), ("c3", 1 << 18, 1 << 20, torch.int64)):
+    wl = datagen.make(cfg, n_r=nr, n_s=ns)
+    want = oracle.join(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload)
+    d = lambda a: torch.from_numpy(np.ascontiguousarray(a)).cuda()
+    with RadixJoin(key_dtype=kdt, radix_passes=2, radix_bits=(8, 8)) as j:
+        r = j.join(d(wl.R.key), d(wl.R.payload), d(wl.S.key), d(wl.S.payload))
+    got = dict(count=r.match_count, sum_r=r.sum_r_payload, sum_s=r.sum_s_payload, checksum=r.pair_checksum)
+    assert got == {k: want[k] for k in got}, (cfg, got, want)
+print("ok")
+'''
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    env = dict(os.environ, HAPE_JOINT="0", PYTHONPATH=root)
+    r = subprocess.run([sys.executable, "-c", code], cwd=root, env=env, capture_output=True, text=True, timeout=600)
+    assert r.returncode == 0 and "ok" in r.stdout, r.stdout + r.stderr
