@@ -12,9 +12,9 @@ function.  DESIGN.md reading R1 fixes it:
 
 and the bit fields of h (reading R3):
   destination GPU  = top g = log2(G) bits of h
-  pass-1 bucket    = bits [0, B1)
-  pass-2 bucket    = bits [B1, B1+B2)
-  partition id     = bits [0, B1+B2) read as p1 + ... i.e. final partition
+  pass-1 bucket    = bits [B2, B2+B1)   (bits [0, B1) for a one-pass plan)
+  pass-2 bucket    = bits [0, B2)
+  partition id     = bits [0, B1+B2), i.e. the final partition
                      q = bucket1 * 2^B2 + bucket2 (pass-1 major)
 
 This module restates those definitions in numpy for the invariant tests; it
@@ -70,7 +70,7 @@ def bits(hv: np.ndarray, lo: int, n: int) -> np.ndarray:
 def partition_id(keys: np.ndarray, b1: int, b2: int, identity: bool = False) -> np.ndarray:
     """Final partition q = bucket1 * 2^b2 + bucket2 (pass-1 major order)."""
     hv = h(keys, identity)
-    return bits(hv, 0, b1) * (1 << b2) + bits(hv, b1, b2)
+    return bits(hv, b2, b1) * (1 << b2) + bits(hv, 0, b2)
 
 
 def destination(keys: np.ndarray, world: int, identity: bool = False) -> np.ndarray:

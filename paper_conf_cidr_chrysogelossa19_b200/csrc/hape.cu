@@ -295,7 +295,7 @@ static hape_status hist_joint_t(hape_join* h, const Src& s, SegMap m, BitField b
     attr_set = true;
   }
   const uint32_t nch = m.nseg * m.cps;
-  kern<<<joint_grid(h, nch), HJ_THREADS, joint_smem(P1, P2), h->stream>>>(s.in, m, bf1, bf2, P1, P2, rowsum, part,
+  kern<<<joint_grid(h, nch), HJ_THREADS, joint_smem(P1, P2), h->stream>>>(s.in, m, P1, P2, rowsum, part,
                                                                         ovf);
   return HAPE_OK;
 }
@@ -536,7 +536,9 @@ static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const
                                         cudaEvent_t side1_ready = nullptr) {
   const int kw = key_width(h->cfg);
   const uint32_t P1 = 1u << pl.bits[0], P2 = 1u << pl.bits[1];
-  const BitField bf1{0u, P1 - 1}, bf2{pl.bits[0], P2 - 1};
+  // DESIGN.md R3: pass 1 takes bits [B2, B2+B1) of h, pass 2 bits [0, B2), so
+  // the final co-partition of a key is the low B1+B2 bits of h
+  const BitField bf1{pl.passes == 2 ? pl.bits[1] : 0u, P1 - 1}, bf2{0u, P2 - 1};
   SegMap m1[2], m2[2];
   Src s2[2];
   for (int s = 0; s < nside; s++) {

@@ -58,7 +58,8 @@ __device__ __forceinline__ uint64_t part_hash(typename UW<KW>::T k) {
   else return fmix64(k);
 }
 
-// bucket = (h >> shift) & mask  (R3: dest = top bits, pass k = low bits)
+// bucket = (h >> shift) & mask  (R3: dest = top bits; pass 2 = bits
+// [0, B2), pass 1 = bits [B2, B2+B1): the final co-partition = low B1+B2 bits)
 struct BitField { uint32_t shift; uint32_t mask; };
 
 __device__ __forceinline__ uint32_t bucket_of(uint64_t h, BitField bf) {
@@ -361,8 +362,7 @@ constexpr int HJ_THREADS = 1024;
 
 template <int KW, int PW, bool AOS, bool IDENT>
 __global__ void __launch_bounds__(HJ_THREADS, 1)
-k_hist_joint(PartIn in, SegMap m, BitField bf1, BitField bf2, uint32_t P1, uint32_t P2,
-             uint32_t* __restrict__ rowsum, uint16_t* __restrict__ part, uint32_t* __restrict__ ovf) {
+k_hist_joint(PartIn in, SegMap m, uint32_t P1, uint32_t P2, uint32_t* __restrict__ rowsum, uint16_t* __restrict__ part, uint32_t* __restrict__ ovf) {
   extern __shared__ __align__(16) uint32_t sh_hj[];
   using K = typename UW<KW>::T;
   using E = typename std::conditional<AOS, Tup<KW, PW>, K>::type;
@@ -379,12 +379,17 @@ k_hist_joint(PartIn in, SegMap m, BitField bf1, BitField bf2, uint32_t P1, uint3
   for (uint32_t i = threadIdx.x; i < QW; i += HJ_THREADS) j16[i] = 0;
   for (uint32_t p = threadIdx.x; p < P1; p += HJ_THREADS) rowtot[p] = 0;
   __syncthreads();
+  // joint bucket = b1 * P2 + b2 = the low B1+B2 bits of h (R3:
+  // pass 1 reads bits [B2, B2+B1), pass 2 bits [0, B2))
+  const uint32_t qmask = Q - 1;
   auto count = [&](K k) {
-    const uint64_t h = part_hash<KW, IDENT>(k);
-    const uint32_t q = bucket_of(h, bf1) * P2 + bucket_of(h, bf2);
-    const uint32_t sh = (q & 1u) * 16;
+    const uint32_t q = (uint32_t)part_hash<KW, IDENT>(k) & qmask;
+    const uint32_t sh = (q & 1u) << 4;
     const uint32_t old = atomicAdd(&j16[q >> 1], 1u << sh);
-    if (((old >> sh) & 0xFFFFu) == 0xFFFFu) {  // this increment wrapped its half
+    // wrap test: the half is 0xFFFF iff (old | ~(0xFFFF << sh)) is all ones;
+    // the rare fix-up runs under a warp-uniform branch
+    const bool wrap = (old | ~(0xFFFFu << sh)) == 0xFFFFFFFFu;
+    if (__any_sync(__activemask(), wrap) && wrap) {  // this increment wrapped its half
       const uint32_t p = q / P2;
       atomicAdd(&ovf[q], 65536u);
       uint32_t dr = 65536u;
@@ -727,9 +732,16 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
       const uint32_t inc = warp_incl_scan(sum);
       if (lane == 31) s_wt[warp] = inc;
       __syncthreads();  // X
-      uint32_t ex = inc - sum;
-      for (int w = 0; w < warp; w++) ex += s_wt[w];
-      for (uint32_t b = b0; b < b1; b++) {
+      // warps past the last bucket have nothing to place (warp-uniform skip);
+      // the others add the totals of the warps before them (one load + a
+      // shuffle scan instead of a loop over the earlier warps)
+      if (warp * 32 * per < P) {
+        constexpr int NW = NT / 32;
+        const uint32_t wt = lane < NW ? s_wt[lane] : 0u;
+        const uint32_t wpre = warp_incl_scan(wt);
+        const uint32_t before = __shfl_sync(0xffffffffu, wpre, (warp + 31) & 31);
+        uint32_t ex = inc - sum + (warp ? before : 0u);
+        for (uint32_t b = b0; b < b1; b++) {
         const uint32_t c = s_cnt[b];
         uint32_t run;
         if constexpr (CLAIM) {
@@ -739,10 +751,11 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
           run = backward ? cur - c : cur;
           s_cur[b] = backward ? cur - c : cur + c;
         }
-        s_st[b] = ex;
-        s_dl[b] = run - ex;
-        s_cnt[b] = 0;
-        ex += c;
+          s_st[b] = ex;
+          s_dl[b] = run - ex;
+          s_cnt[b] = 0;
+          ex += c;
+        }
       }
     }
     __syncthreads();  // B: run starts known
