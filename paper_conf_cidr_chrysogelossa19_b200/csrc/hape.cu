@@ -413,9 +413,19 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a, uint32_t* ctas
   int per_sm = 0;
   CK(h, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, JN_THREADS, smem));
   if (per_sm < 1) return fail(h, HAPE_ERR_UNSUPPORTED, "build+probe does not fit: smem %zu", smem);
+  // plan.slot_bits is the minimum table size: one more bit (shorter chains)
+  // when the larger head array costs no occupancy (register-limited kernels)
+  JoinArgs a2 = a;
+  if (a.slot_bits < 14) {
+    const size_t smem2 = join_smem_bytes<KW, PRW>(a.cap, a.slot_bits + 1);
+    int per_sm2 = 0;
+    CK(h, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm2, kern, JN_THREADS, smem2));
+    if (per_sm2 == per_sm) { a2.slot_bits = a.slot_bits + 1; }
+  }
+  const size_t smem_used = join_smem_bytes<KW, PRW>(a2.cap, a2.slot_bits);
   const unsigned grid = (unsigned)(per_sm * h->num_sms);
   *ctas_out = grid;
-  kern<<<grid, JN_THREADS, smem, h->stream>>>(a);
+  kern<<<grid, JN_THREADS, smem_used, h->stream>>>(a2);
   CK_LAUNCH(h);
   return HAPE_OK;
 }
@@ -500,7 +510,7 @@ static CallLayout layout_for(const hape_join* h, const hape_plan& pl, uint64_t n
       S.cps2 = cps_for(h, ns[s], (uint32_t)P1);
       S.hist2 = cv.take(Q * 4);
       S.bounds2 = cv.take((Q + 1) * 4);
-      S.nparts = joint_grid(h, S.cps1);
+      S.nparts = joint_grid(h, (uint32_t)std::min<uint64_t>(ns[s] / 1024 + 1, 1u << 20));
       S.part = cv.take((size_t)S.nparts * Q * 2);
     } else if (pl.passes == 2) {
       S.cps2 = cps_for(h, ns[s], (uint32_t)P1);
@@ -553,8 +563,11 @@ static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const
   // spilled counts (both zeroed per call).
   const bool joint = use_joint(pl);
   auto hist1 = [&](int s) {
+    // the persistent joint-histogram CTAs take one contiguous range each (the
+    // claiming scatters do not depend on the histogram's chunking)
     if (joint)
-      return launch_hist_joint(h, kw, io[s].in, m1[s], bf1, bf2, P1, P2, at<uint32_t>(h, L.side[s].rowsum1),
+      return launch_hist_joint(h, kw, io[s].in, SegMap{nullptr, 1u, L.side[s].nparts, io[s].in.n}, bf1, bf2, P1, P2,
+                               at<uint32_t>(h, L.side[s].rowsum1),
                                at<uint16_t>(h, L.side[s].part), at<uint32_t>(h, L.side[s].rowsum2));
     return launch_hist(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1));
   };
