@@ -175,6 +175,8 @@ def main():
     ap.add_argument("--no-mat", action="store_true", help="c3 without materialised pairs (diagnostics)")
     ap.add_argument("--bag", action="store_true",
                     help="do not declare R's keys unique (HAPE_FLAG_R_UNIQUE): full bag-semantics probe")
+    ap.add_argument("--no-ablation", action="store_true",
+                    help="skip the non-partitioned GPU join comparison (PAPER.md Fig. 6)")
     ap.add_argument("--exchange", action="store_true",
                     help="at N=1, run the device-partition + NCCL exchange path through a 1-rank communicator")
     args = ap.parse_args()
@@ -348,6 +350,28 @@ def main():
                "h2d_stage_ms": r2.stage_ms.get("h2d")}
         del hk, ho
 
+    # ---- PAPER.md Fig. 6's comparison on this hardware: the non-partitioned
+    # GPU hash join (one HBM table over R; hape_nonpartitioned_join) on the
+    # same resident inputs, same result
+    nonpart = None
+    if world == 1 and not args.exchange and not args.no_ablation:
+        for _ in range(2):
+            rn = j.join_nonpartitioned(rk, rp, sk, sp, out_r, out_s)
+        barrier()
+        e0.record(stream)
+        n_np = max(1, min(args.steps, 5))
+        for _ in range(n_np):
+            rn = j.join_nonpartitioned(rk, rp, sk, sp, out_r, out_s)
+        e1.record(stream)
+        barrier()
+        np_ms = e0.elapsed_time(e1) / n_np
+        nonpart = {"method": "non-partitioned GPU hash join (hape_nonpartitioned_join, PAPER.md Fig. 6 baseline)",
+                   "ms_per_step": round(np_ms, 4), "value": total_tuples / (np_ms / 1000.0), "unit": UNIT,
+                   "radix_speedup": round(np_ms / ms, 3),
+                   "stages_ms": {"build (clear + insert)": round(rn.stage_ms["np_build"], 4),
+                                 "probe": round(rn.stage_ms["np_probe"], 4)},
+                   "same_result_as_radix": rn.as_tuple() == res.as_tuple()}
+
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
         try:
@@ -375,6 +399,8 @@ def main():
             "e2e": e2e,
             "cpu_baseline": cpu,
         }
+        if nonpart is not None:
+            line["nonpartitioned_gpu"] = nonpart
         if verify is not None:
             line["verified_vs_provenance"] = verify
         print(json.dumps(line), flush=True)

@@ -20,10 +20,11 @@ from ._lib import (HAPE_INT32, HAPE_INT64, HAPE_MEM_DEVICE, HAPE_MEM_HOST, HAPE_
                    HAPE_ERR_OUTPUT_CAPACITY, HAPE_PART_HASH, HAPE_PART_IDENTITY, STAGES,
                    hape_join_config, hape_join_create, hape_join_destroy, hape_join_plan,
                    hape_join_result, hape_last_error, hape_output, hape_radix_join,
+                   hape_nonpartitioned_join,
                    hape_relation, hape_status_string, hape_debug_partition, hape_version)
 
 __all__ = ["RadixJoin", "JoinResult", "HapeError", "hape_version", "hape_join_create",
-           "hape_radix_join", "hape_join_destroy", "STAGES"]
+           "hape_radix_join", "hape_nonpartitioned_join", "hape_join_destroy", "STAGES"]
 
 
 class HapeError(RuntimeError):
@@ -148,6 +149,16 @@ class RadixJoin:
             cur.synchronize()
 
     def join(self, rk, rp, sk, sp, out_r=None, out_s=None, raise_on_capacity: bool = True) -> JoinResult:
+        """hape_radix_join: the partitioned radix hash join (the product path)."""
+        return self._call(hape_radix_join, rk, rp, sk, sp, out_r, out_s, raise_on_capacity)
+
+    def join_nonpartitioned(self, rk, rp, sk, sp, out_r=None, out_s=None,
+                            raise_on_capacity: bool = True) -> JoinResult:
+        """hape_nonpartitioned_join: one HBM hash table over R (Fig. 6's
+        non-partitioned GPU join, kept for the comparison)."""
+        return self._call(hape_nonpartitioned_join, rk, rp, sk, sp, out_r, out_s, raise_on_capacity)
+
+    def _call(self, fn, rk, rp, sk, sp, out_r, out_s, raise_on_capacity) -> JoinResult:
         self._order_inputs()
         R = _rel(rk, rp)
         S = _rel(sk, sp)
@@ -158,7 +169,7 @@ class RadixJoin:
             out = hape_output(out_r.data_ptr(), out_s.data_ptr(), out_r.shape[0],
                               HAPE_MEM_DEVICE if out_r.is_cuda else HAPE_MEM_HOST)
         res = hape_join_result()
-        st = hape_radix_join(self._h, R, S, out, res)
+        st = fn(self._h, R, S, out, res)
         if st != HAPE_OK and not (st == HAPE_ERR_OUTPUT_CAPACITY and not raise_on_capacity):
             raise HapeError(st, hape_last_error(self._h))
         return JoinResult(

@@ -29,13 +29,13 @@ HAPE_MEM_HOST = 1
 HAPE_FLAG_R_UNIQUE = 1
 
 STAGES = ["h2d", "devpart", "exchange", "hist1", "scan1", "scatter1", "hist2", "scan2",
-          "scatter2", "worklist", "build_probe", "finalize", "total"]
+          "scatter2", "worklist", "build_probe", "np_build", "np_probe", "finalize", "total"]
 HAPE_NSTAGES = len(STAGES)
 
 EXPORTED = ["hape_version", "hape_status_string", "hape_join_create", "hape_radix_join",
             "hape_join_destroy", "hape_last_error", "hape_join_plan", "hape_debug_partition",
             "hape_nccl_unique_id", "hape_nccl_comm_init", "hape_nccl_comm_destroy",
-            "hape_exchange_plan"]
+            "hape_exchange_plan", "hape_nonpartitioned_join"]
 
 
 class hape_join_config(ctypes.Structure):
@@ -93,6 +93,9 @@ def _load() -> ctypes.CDLL:
     lib.hape_radix_join.restype = ctypes.c_int
     lib.hape_radix_join.argtypes = [vp, P(hape_relation), P(hape_relation), P(hape_output),
                                     P(hape_join_result)]
+    lib.hape_nonpartitioned_join.restype = ctypes.c_int
+    lib.hape_nonpartitioned_join.argtypes = [vp, P(hape_relation), P(hape_relation), P(hape_output),
+                                             P(hape_join_result)]
     lib.hape_join_destroy.restype = ctypes.c_int
     lib.hape_join_destroy.argtypes = [vp]
     lib.hape_last_error.restype = ctypes.c_char_p
@@ -135,6 +138,11 @@ def hape_join_create(cfg: hape_join_config):
 def hape_radix_join(h, R: hape_relation, S: hape_relation, out, res: hape_join_result) -> int:
     return lib.hape_radix_join(h, ctypes.byref(R), ctypes.byref(S),
                                ctypes.byref(out) if out is not None else None, ctypes.byref(res))
+
+
+def hape_nonpartitioned_join(h, R: hape_relation, S: hape_relation, out, res: hape_join_result) -> int:
+    return lib.hape_nonpartitioned_join(h, ctypes.byref(R), ctypes.byref(S),
+                                        ctypes.byref(out) if out is not None else None, ctypes.byref(res))
 
 
 def hape_join_destroy(h) -> int:

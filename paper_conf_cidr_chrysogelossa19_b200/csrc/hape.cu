@@ -25,6 +25,7 @@
 
 #include "hape.h"
 #include "kernels.cuh"
+#include "nonpart.cuh"
 
 using namespace hape;
 
@@ -70,6 +71,7 @@ struct hape_join {
   DevBuf recv[2];         // G>1 exchange receive buffers
   DevBuf outst[2];        // host-output staging
   DevBuf small;           // histograms, bounds, work list, counters
+  DevBuf np_table;        // hape_nonpartitioned_join: the HBM hash table
   unsigned long long* h_res = nullptr;  // pinned: acc[4], out_ctr, (n_items | item_ctr)
   // cached CUDA graph of the local join sequence (keyed by pointers + sizes)
   cudaGraphExec_t gexec = nullptr;
@@ -742,6 +744,25 @@ static hape_status exchange(hape_join* h, Src in[2], Src out[2]) {
   return HAPE_OK;
 }
 
+// stage times after the final event: each used stage runs until the next
+// used stage mark (stages are marked in enum order on the join stream)
+static void stage_times(hape_join* h, hape_join_result* res) {
+  int order[HAPE_NSTAGES];
+  int no = 0;
+  for (int s = HAPE_STAGE_H2D; s < HAPE_STAGE_TOTAL; s++)
+    if (h->ev_used[s]) order[no++] = s;
+  for (int i = 0; i < no; i++) {
+    cudaEvent_t end = i + 1 < no ? h->ev[order[i + 1]] : h->ev[HAPE_NSTAGES];
+    float ms = 0;
+    cudaEventElapsedTime(&ms, h->ev[order[i]], end);
+    res->stage_ms[order[i]] = ms;
+  }
+  float tot = 0;
+  cudaEventElapsedTime(&tot, h->ev[HAPE_STAGE_TOTAL], h->ev[HAPE_NSTAGES]);
+  res->stage_ms[HAPE_STAGE_TOTAL] = tot;
+  (void)cudaGetLastError();
+}
+
 // ---------------------------------------------------------------------------
 // the join
 // ---------------------------------------------------------------------------
@@ -908,21 +929,125 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   cudaEventRecord(h->ev[HAPE_NSTAGES], h->stream);
   CK(h, cudaStreamSynchronize(h->stream));
   res->kernel_launches = h->launches;
-  // stage times: each used stage runs until the next used stage mark
-  int order[HAPE_NSTAGES];
-  int no = 0;
-  for (int s = HAPE_STAGE_H2D; s < HAPE_STAGE_TOTAL; s++)
-    if (h->ev_used[s]) order[no++] = s;
-  for (int i = 0; i < no; i++) {
-    cudaEvent_t end = i + 1 < no ? h->ev[order[i + 1]] : h->ev[HAPE_NSTAGES];
-    float ms = 0;
-    cudaEventElapsedTime(&ms, h->ev[order[i]], end);
-    res->stage_ms[order[i]] = ms;
+  stage_times(h, res);
+  if (mat && r[4] > out->capacity)
+    return fail(h, HAPE_ERR_OUTPUT_CAPACITY, "join produced %llu pairs > capacity %llu", (unsigned long long)r[4],
+                (unsigned long long)out->capacity);
+  return HAPE_OK;
+}
+
+// ---------------------------------------------------------------------------
+// the non-partitioned GPU hash join (Fig. 6's baseline; nonpart.cuh)
+// ---------------------------------------------------------------------------
+template <int KW, int PRW, int PSW>
+static hape_status np_launch(hape_join* h, const Src& r, const Src& s, void* table, uint32_t mask, bool mat,
+                             void* mat_r, void* mat_s, unsigned long long cap, unsigned long long* acc,
+                             unsigned long long* out_ctr) {
+  using K = typename UW<KW>::T;
+  auto* tab = static_cast<NpSlot<KW, PRW>*>(table);
+  mark(h, HAPE_STAGE_NP_BUILD);
+  CK(h, cudaMemsetAsync(table, 0, ((size_t)mask + 1) * sizeof(NpSlot<KW, PRW>), h->stream));
+  const unsigned gmax = (unsigned)h->num_sms * 8;
+  if (r.n) {
+    k_np_build<KW, PRW><<<std::min<unsigned>(gmax, (r.n + NP_THREADS - 1) / NP_THREADS), NP_THREADS, 0, h->stream>>>(
+        static_cast<const K*>(r.in.k), static_cast<const typename UW<PRW>::T*>(r.in.p), r.n, tab, mask);
+    CK_LAUNCH(h);
   }
-  float tot = 0;
-  cudaEventElapsedTime(&tot, h->ev[HAPE_STAGE_TOTAL], h->ev[HAPE_NSTAGES]);
-  res->stage_ms[HAPE_STAGE_TOTAL] = tot;
-  (void)cudaGetLastError();
+  mark(h, HAPE_STAGE_NP_PROBE);
+  if (s.n) {
+    const unsigned grid = std::min<unsigned>(gmax, (s.n + NP_THREADS - 1) / NP_THREADS);
+    const uint32_t uq = (h->cfg.flags & HAPE_FLAG_R_UNIQUE) ? 1u : 0u;
+    const auto* sk = static_cast<const K*>(s.in.k);
+    const auto* sp = static_cast<const typename UW<PSW>::T*>(s.in.p);
+    if (mat)
+      k_np_probe<KW, PRW, PSW, true><<<grid, NP_THREADS, 0, h->stream>>>(sk, sp, s.n, tab, mask, uq, acc, mat_r,
+                                                                         mat_s, cap, out_ctr);
+    else
+      k_np_probe<KW, PRW, PSW, false><<<grid, NP_THREADS, 0, h->stream>>>(sk, sp, s.n, tab, mask, uq, acc, nullptr,
+                                                                          nullptr, 0, out_ctr);
+    CK_LAUNCH(h);
+  }
+  return HAPE_OK;
+}
+
+static hape_status np_join_impl(hape_join* h, const hape_relation* R, const hape_relation* S, const hape_output* out,
+                                hape_join_result* res) {
+  const hape_join_config& c = h->cfg;
+  const int kw = key_width(c), prw = pay_width(c.r_payload_type), psw = pay_width(c.s_payload_type);
+  CKS(check_rel(h, R, kw, prw, "R"));
+  CKS(check_rel(h, S, kw, psw, "S"));
+  if (c.world_size > 1 || h->comm)
+    return fail(h, HAPE_ERR_UNSUPPORTED, "the non-partitioned join is single-GPU (world_size 1)");
+  if (R->n > (1ull << 30)) return fail(h, HAPE_ERR_UNSUPPORTED, "non-partitioned join: |R| > 2^30");
+  const bool mat = out && out->capacity > 0;
+  if (mat) {
+    if (!out->r_payload || !out->s_payload) return fail(h, HAPE_ERR_INVALID_ARG, "output buffers NULL");
+    if (out->mem != HAPE_MEM_DEVICE && out->mem != HAPE_MEM_HOST) return fail(h, HAPE_ERR_INVALID_ARG, "out.mem");
+  }
+  CK(h, cudaSetDevice(h->dev));
+  memset(res, 0, sizeof *res);
+  for (int i = 0; i < HAPE_NSTAGES; i++) h->ev_used[i] = false;
+  h->launches = 0;
+  mark(h, HAPE_STAGE_TOTAL);
+  mark(h, HAPE_STAGE_H2D);
+  Src in[2];
+  CKS(stage_in(h, R, kw, prw, h->stage[0], h->stage[1], &in[0]));
+  CKS(stage_in(h, S, kw, psw, h->stage[2], h->stage[3], &in[1]));
+  const uint32_t tbits = std::max<uint32_t>(10, ceil_log2_u64(2 * std::max<uint64_t>(R->n, 1)));
+  const size_t slot = (kw == 4) ? 16 : 32;
+  CKS(ensure(h, h->np_table, ((size_t)1 << tbits) * slot));
+  CKS(ensure(h, h->small, 64));
+  unsigned long long* acc = at<unsigned long long>(h, 0);
+  unsigned long long* out_ctr = acc + 4;
+  CK(h, cudaMemsetAsync(acc, 0, 5 * 8, h->stream));
+  void* mat_r = nullptr;
+  void* mat_s = nullptr;
+  if (mat) {
+    mat_r = out->r_payload;
+    mat_s = out->s_payload;
+    if (out->mem == HAPE_MEM_HOST) {
+      CKS(ensure(h, h->outst[0], out->capacity * prw));
+      CKS(ensure(h, h->outst[1], out->capacity * psw));
+      mat_r = h->outst[0].p;
+      mat_s = h->outst[1].p;
+    }
+  }
+  const uint32_t mask = (1u << tbits) - 1;
+  const unsigned long long cap = mat ? out->capacity : 0;
+  void* tab = h->np_table.p;
+#define HAPE_NP(KW, PRW, PSW) np_launch<KW, PRW, PSW>(h, in[0], in[1], tab, mask, mat, mat_r, mat_s, cap, acc, out_ctr)
+  hape_status st;
+  if (kw == 4) {
+    if (prw == 4) st = psw == 4 ? HAPE_NP(4, 4, 4) : HAPE_NP(4, 4, 8);
+    else st = psw == 4 ? HAPE_NP(4, 8, 4) : HAPE_NP(4, 8, 8);
+  } else {
+    if (prw == 4) st = psw == 4 ? HAPE_NP(8, 4, 4) : HAPE_NP(8, 4, 8);
+    else st = psw == 4 ? HAPE_NP(8, 8, 4) : HAPE_NP(8, 8, 8);
+  }
+#undef HAPE_NP
+  CKS(st);
+  mark(h, HAPE_STAGE_FINALIZE);
+  CK(h, cudaMemcpyAsync(h->h_res, acc, 5 * 8, cudaMemcpyDeviceToHost, h->stream));
+  CK(h, cudaStreamSynchronize(h->stream));
+  const unsigned long long* r = h->h_res;
+  res->match_count = res->local_match_count = r[0];
+  res->sum_r_payload = res->local_sum_r = r[1];
+  res->sum_s_payload = res->local_sum_s = r[2];
+  res->pair_checksum = res->local_pair_checksum = r[3];
+  res->n_required = r[0];
+  res->n_written = mat ? std::min<uint64_t>(r[4], out->capacity) : 0;
+  res->r_local = R->n;
+  res->s_local = S->n;
+  res->passes = 0;
+  res->n_partitions = 1;
+  if (mat && out->mem == HAPE_MEM_HOST && res->n_written) {
+    CK(h, cudaMemcpyAsync(out->r_payload, mat_r, res->n_written * prw, cudaMemcpyDeviceToHost, h->stream));
+    CK(h, cudaMemcpyAsync(out->s_payload, mat_s, res->n_written * psw, cudaMemcpyDeviceToHost, h->stream));
+  }
+  cudaEventRecord(h->ev[HAPE_NSTAGES], h->stream);
+  CK(h, cudaStreamSynchronize(h->stream));
+  res->kernel_launches = h->launches;
+  stage_times(h, res);
   if (mat && r[4] > out->capacity)
     return fail(h, HAPE_ERR_OUTPUT_CAPACITY, "join produced %llu pairs > capacity %llu", (unsigned long long)r[4],
                 (unsigned long long)out->capacity);
@@ -934,7 +1059,7 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
 // ---------------------------------------------------------------------------
 extern "C" {
 
-const char* hape_version(void) { return "hape-b200 1.0 (sm_100a, ABI 1)"; }
+const char* hape_version(void) { return "hape-b200 1.1 (sm_100a, ABI 2)"; }
 
 const char* hape_status_string(hape_status s) {
   switch (s) {
@@ -1023,6 +1148,7 @@ hape_status hape_join_destroy(hape_join* h) {
     if (b.p) cudaFree(b.p);
   if (h->gexec) cudaGraphExecDestroy(h->gexec);
   if (h->small.p) cudaFree(h->small.p);
+  if (h->np_table.p) cudaFree(h->np_table.p);
   if (h->h_res) cudaFreeHost(h->h_res);
   if (h->h_bounds) cudaFreeHost(h->h_bounds);
   for (auto& e : h->ev)
@@ -1048,6 +1174,17 @@ hape_status hape_radix_join(hape_join* h, const hape_relation* R, const hape_rel
   if (!res) return fail(h, HAPE_ERR_INVALID_ARG, "res is NULL");
   try {
     return join_impl(h, R, S, out, res);
+  } catch (...) {
+    return fail(h, HAPE_ERR_CUDA, "unexpected C++ exception");
+  }
+}
+
+hape_status hape_nonpartitioned_join(hape_join* h, const hape_relation* R, const hape_relation* S,
+                                     const hape_output* out, hape_join_result* res) {
+  if (!h) return HAPE_ERR_INVALID_ARG;
+  if (!res) return fail(h, HAPE_ERR_INVALID_ARG, "res is NULL");
+  try {
+    return np_join_impl(h, R, S, out, res);
   } catch (...) {
     return fail(h, HAPE_ERR_CUDA, "unexpected C++ exception");
   }
