@@ -11,9 +11,10 @@ kill $SMI
 B="python bench.py --config $CFG --steps 1 --warmup 3 --no-e2e --no-cpu-baseline"
 timeout 600 ncu --metrics gpu__time_duration.sum,dram__bytes_read.sum,dram__bytes_write.sum --clock-control none --csv --log-file gpurun_out/launches_${TAG}_${CFG}.csv $B > /dev/null 2>&1
 # per-launch skip counts: 3 warm-up steps precede the profiled one
-NH=$((3*4)); NS=$((3*4)); NB=3
-if [ "$CFG" = "c1" ]; then NH=6; NS=6; fi
-for K in k_hist:$NH k_scatter:$NS k_build_probe:$NB; do
+# (two-pass plans: one joint histogram per relation and step, 4 scatters)
+NH=$((3*2)); NS=$((3*4)); NB=3; HK=k_hist_joint
+if [ "$CFG" = "c1" ]; then NH=6; NS=6; HK=k_hist; fi
+for K in $HK:$NH k_scatter:$NS k_build_probe:$NB; do
   N=${K%%:*}; S=${K##*:}
   timeout 600 ncu --set full --clock-control none --import-source on -k regex:$N -s $S -c 1 -o gpurun_out/full_${TAG}_${CFG}_${N} $B > /dev/null 2>&1
 done
