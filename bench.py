@@ -177,6 +177,10 @@ def main():
                     help="do not declare R's keys unique (HAPE_FLAG_R_UNIQUE): full bag-semantics probe")
     ap.add_argument("--no-ablation", action="store_true",
                     help="skip the non-partitioned GPU join comparison (PAPER.md Fig. 6)")
+    ap.add_argument("--no-coprocess", action="store_true",
+                    help="skip the out-of-HBM co-processing measurement (hape_coprocess_join, PAPER.md Fig. 7)")
+    ap.add_argument("--cp-fanout", type=int, default=3,
+                    help="co-processing: host fan-out bits (F = 2^bits co-partition pairs, each one transfer)")
     ap.add_argument("--exchange", action="store_true",
                     help="at N=1, run the device-partition + NCCL exchange path through a 1-rank communicator")
     args = ap.parse_args()
@@ -326,6 +330,7 @@ def main():
 
     # ---- end to end through the same C ABI call with pinned host buffers
     e2e = None
+    coproc = None
     if not args.no_e2e:
         hk = [x.cpu().pin_memory() for x in (rk, rp, sk, sp)]
         ho = None
@@ -348,6 +353,37 @@ def main():
         e2e = {"value": total_tuples / (e_ms / 1000.0), "unit": UNIT, "ms_per_step": e_ms,
                "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h // n_e2e,
                "h2d_stage_ms": r2.stage_ms.get("h2d")}
+        # ---- PAPER.md §5 / Fig. 7 co-processing on the same host-resident
+        # inputs: CPU-side co-partitioning into F pairs, one transfer per pair
+        # overlapping the previous pair's device join (hape_coprocess_join,
+        # SURVEY §8.f NEXT-3).  Wall-clock timed: the call includes host work.
+        if world == 1 and not args.exchange and not args.no_coprocess:
+            for _ in range(2):
+                rc = j.coprocess_join(*hk, *(ho or (None, None)), fanout_bits=args.cp_fanout)
+            n_cp = 3
+            t0 = time.perf_counter()
+            agg = {}
+            for _ in range(n_cp):
+                rc = j.coprocess_join(*hk, *(ho or (None, None)), fanout_bits=args.cp_fanout)
+                for k, v in rc.stage_ms.items():
+                    agg[k] = agg.get(k, 0.0) + v / n_cp
+            cp_ms = (time.perf_counter() - t0) * 1000.0 / n_cp
+            # PCIe H2D bandwidth as this call measured it: its bytes over the
+            # summed copy-stream transfer time of the co-partition pairs
+            pcie_gbs = h2d / (agg["h2d"] / 1000.0) / 1e9 if agg.get("h2d") else None
+            dev = sum(v for k, v in agg.items() if k not in ("h2d", "host_part", "total"))
+            coproc = {
+                "method": "hape_coprocess_join: CPU co-partitioning (host threads, pinned) + one H2D per pair + device radix join per pair",
+                "fanout": rc.n_partitions, "host_threads": os.cpu_count(),
+                "ms_per_step": round(cp_ms, 3), "value": total_tuples / (cp_ms / 1000.0), "unit": UNIT,
+                "stages_ms": {"host_partition": round(agg.get("host_part", 0), 3),
+                              "h2d (copy stream)": round(agg.get("h2d", 0), 3),
+                              "device joins": round(dev, 3)},
+                # host-link roofline: every input byte crosses PCIe once (the
+                # point of the plan, P723-724); frac = that transfer time / step
+                "pcie_roofline": {"bytes": h2d, "h2d_GB/s_measured": round(pcie_gbs, 1) if pcie_gbs else None,
+                                  "frac": round((h2d / (pcie_gbs * 1e9) * 1000.0) / cp_ms, 3) if pcie_gbs else None},
+                "same_result_as_radix": rc.as_tuple() == res.as_tuple()}
         del hk, ho
 
     # ---- PAPER.md Fig. 6's comparison on this hardware: the non-partitioned
@@ -401,6 +437,8 @@ def main():
         }
         if nonpart is not None:
             line["nonpartitioned_gpu"] = nonpart
+        if coproc is not None:
+            line["coprocess"] = coproc
         if verify is not None:
             line["verified_vs_provenance"] = verify
         print(json.dumps(line), flush=True)

@@ -20,11 +20,13 @@ from ._lib import (HAPE_INT32, HAPE_INT64, HAPE_MEM_DEVICE, HAPE_MEM_HOST, HAPE_
                    HAPE_ERR_OUTPUT_CAPACITY, HAPE_PART_HASH, HAPE_PART_IDENTITY, STAGES,
                    hape_join_config, hape_join_create, hape_join_destroy, hape_join_plan,
                    hape_join_result, hape_last_error, hape_output, hape_radix_join,
-                   hape_nonpartitioned_join,
+                   hape_nonpartitioned_join, hape_coprocess_join, hape_coprocess_config,
+                   hape_host_partition,
                    hape_relation, hape_status_string, hape_debug_partition, hape_version)
 
 __all__ = ["RadixJoin", "JoinResult", "HapeError", "hape_version", "hape_join_create",
-           "hape_radix_join", "hape_nonpartitioned_join", "hape_join_destroy", "STAGES"]
+           "hape_radix_join", "hape_nonpartitioned_join", "hape_coprocess_join", "hape_join_destroy",
+           "host_partition", "STAGES"]
 
 
 class HapeError(RuntimeError):
@@ -158,6 +160,17 @@ class RadixJoin:
         non-partitioned GPU join, kept for the comparison)."""
         return self._call(hape_nonpartitioned_join, rk, rp, sk, sp, out_r, out_s, raise_on_capacity)
 
+    def coprocess_join(self, rk, rp, sk, sp, out_r=None, out_s=None, device_budget: int = 0,
+                       fanout_bits: int = 0, host_threads: int = 0,
+                       raise_on_capacity: bool = True) -> JoinResult:
+        """hape_coprocess_join: out-of-HBM co-processing of host-resident R and S
+        (CPU tensors, pinned for full PCIe speed): CPU-side co-partitioning, one
+        transfer per co-partition pair, the device radix join per pair (PAPER.md
+        §5, P717-737; Fig. 7).  stage_ms['host_part'] is the host step."""
+        cp = hape_coprocess_config(int(device_budget), int(fanout_bits), int(host_threads))
+        fn = lambda h, R, S, out, res: hape_coprocess_join(h, R, S, cp, out, res)  # noqa: E731
+        return self._call(fn, rk, rp, sk, sp, out_r, out_s, raise_on_capacity)
+
     def _call(self, fn, rk, rp, sk, sp, out_r, out_s, raise_on_capacity) -> JoinResult:
         self._order_inputs()
         R = _rel(rk, rp)
@@ -200,3 +213,23 @@ class RadixJoin:
         if st != HAPE_OK:
             raise HapeError(st, hape_last_error(self._h))
         return ok, op, ob.to(torch.int64) & 0xFFFFFFFF, pout
+
+
+def host_partition(key, pay, fanout_bits: int, identity: bool = False, threads: int = 0):
+    """hape_host_partition (the co-processing join's CPU step) on CPU tensors:
+    returns (keys, payloads, bounds[int64 of 2^fanout_bits + 1])."""
+    import torch
+    if key.is_cuda or pay.is_cuda:
+        raise ValueError("host_partition takes CPU tensors")
+    key, pay = key.contiguous(), pay.contiguous()
+    rel = _rel(key, pay)
+    ok = torch.empty_like(key)
+    op = torch.empty_like(pay)
+    F = 1 << int(fanout_bits)
+    b = (ctypes.c_uint64 * (F + 1))()
+    st = hape_host_partition(rel, _dt(key.dtype), _dt(pay.dtype),
+                             HAPE_PART_IDENTITY if identity else HAPE_PART_HASH, int(fanout_bits), int(threads),
+                             ok.data_ptr() if ok.numel() else None, op.data_ptr() if op.numel() else None, b)
+    if st != HAPE_OK:
+        raise HapeError(st, "hape_host_partition failed")
+    return ok, op, torch.tensor(list(b), dtype=torch.int64)

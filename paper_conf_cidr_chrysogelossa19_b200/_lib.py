@@ -29,13 +29,14 @@ HAPE_MEM_HOST = 1
 HAPE_FLAG_R_UNIQUE = 1
 
 STAGES = ["h2d", "devpart", "exchange", "hist1", "scan1", "scatter1", "hist2", "scan2",
-          "scatter2", "worklist", "build_probe", "np_build", "np_probe", "finalize", "total"]
+          "scatter2", "worklist", "build_probe", "np_build", "np_probe", "finalize", "host_part", "total"]
 HAPE_NSTAGES = len(STAGES)
 
 EXPORTED = ["hape_version", "hape_status_string", "hape_join_create", "hape_radix_join",
             "hape_join_destroy", "hape_last_error", "hape_join_plan", "hape_debug_partition",
             "hape_nccl_unique_id", "hape_nccl_comm_init", "hape_nccl_comm_destroy",
-            "hape_exchange_plan", "hape_nonpartitioned_join"]
+            "hape_exchange_plan", "hape_nonpartitioned_join", "hape_coprocess_join",
+            "hape_host_partition"]
 
 
 class hape_join_config(ctypes.Structure):
@@ -69,6 +70,11 @@ class hape_join_result(ctypes.Structure):
                 ("kernel_launches", ctypes.c_uint32), ("stage_ms", ctypes.c_float * HAPE_NSTAGES)]
 
 
+class hape_coprocess_config(ctypes.Structure):
+    _fields_ = [("device_budget", ctypes.c_uint64), ("fanout_bits", ctypes.c_uint32),
+                ("host_threads", ctypes.c_int)]
+
+
 class hape_plan(ctypes.Structure):
     _fields_ = [("passes", ctypes.c_uint32), ("bits", ctypes.c_uint32 * 2),
                 ("slot_bits", ctypes.c_uint32), ("slot_shift", ctypes.c_uint32),
@@ -96,6 +102,12 @@ def _load() -> ctypes.CDLL:
     lib.hape_nonpartitioned_join.restype = ctypes.c_int
     lib.hape_nonpartitioned_join.argtypes = [vp, P(hape_relation), P(hape_relation), P(hape_output),
                                              P(hape_join_result)]
+    lib.hape_coprocess_join.restype = ctypes.c_int
+    lib.hape_coprocess_join.argtypes = [vp, P(hape_relation), P(hape_relation), P(hape_coprocess_config),
+                                        P(hape_output), P(hape_join_result)]
+    lib.hape_host_partition.restype = ctypes.c_int
+    lib.hape_host_partition.argtypes = [P(hape_relation), ctypes.c_int, ctypes.c_int, ctypes.c_int,
+                                        ctypes.c_uint32, ctypes.c_int, vp, vp, P(ctypes.c_uint64)]
     lib.hape_join_destroy.restype = ctypes.c_int
     lib.hape_join_destroy.argtypes = [vp]
     lib.hape_last_error.restype = ctypes.c_char_p
@@ -143,6 +155,18 @@ def hape_radix_join(h, R: hape_relation, S: hape_relation, out, res: hape_join_r
 def hape_nonpartitioned_join(h, R: hape_relation, S: hape_relation, out, res: hape_join_result) -> int:
     return lib.hape_nonpartitioned_join(h, ctypes.byref(R), ctypes.byref(S),
                                         ctypes.byref(out) if out is not None else None, ctypes.byref(res))
+
+
+def hape_coprocess_join(h, R: hape_relation, S: hape_relation, cp, out, res: hape_join_result) -> int:
+    return lib.hape_coprocess_join(h, ctypes.byref(R), ctypes.byref(S),
+                                   ctypes.byref(cp) if cp is not None else None,
+                                   ctypes.byref(out) if out is not None else None, ctypes.byref(res))
+
+
+def hape_host_partition(rel: hape_relation, key_type: int, payload_type: int, part_fn: int,
+                        fanout_bits: int, threads: int, out_keys: int, out_payloads: int, out_bounds) -> int:
+    return lib.hape_host_partition(ctypes.byref(rel), key_type, payload_type, part_fn, fanout_bits, threads,
+                                   out_keys, out_payloads, out_bounds)
 
 
 def hape_join_destroy(h) -> int:

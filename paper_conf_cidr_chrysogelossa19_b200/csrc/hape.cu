@@ -80,6 +80,13 @@ struct hape_join {
   bool g_ev_used[HAPE_NSTAGES] = {};
   uint32_t* h_bounds = nullptr;         // pinned: gathered device-partition bounds
   size_t h_bounds_cap = 0;
+  // hape_coprocess_join: pinned host co-partitions (R key, R pay, S key, S
+  // pay), two device staging sets, copy events (start, end) per set
+  void* hp[4] = {};
+  size_t hp_cap[4] = {};
+  DevBuf cpst[2][4];
+  cudaEvent_t ev_h2d[2][2] = {};
+  bool in_coprocess = false;            // join_impl: no CUDA-graph capture (sizes change per call)
 };
 
 // ---------------------------------------------------------------------------
@@ -403,38 +410,77 @@ static hape_status launch_scatter(hape_join* h, int kw, const Src& s, SegMap m, 
 #undef HAPE_SC_DISPATCH
 }
 
-template <int KW, int PRW, int PSW, bool MAT>
-static hape_status launch_join_t(hape_join* h, const JoinArgs& a, uint32_t* ctas_out) {
-  auto kern = k_build_probe<KW, PRW, PSW, MAT>;
-  const size_t smem = join_smem_bytes<KW, PRW>(a.cap, a.slot_bits);
+// Build+probe shape: SR kernels (SU > 0) stage S through a smem tile ring of
+// SU*256-tuple tiles (the materialising and 16-byte-tuple forms, whose probe
+// cannot keep a software-pipelined S batch in registers); the others read S
+// straight from HBM with a register-pipelined batch.  HAPE_JN_SU=0/1/2/4
+// forces the form, HAPE_JN_NRB / HAPE_JN_NSB the ring depths (tuning only).
+static int env_int(const char* name, int dflt) {
+  const char* e = getenv(name);
+  return e ? atoi(e) : dflt;
+}
+
+template <int KW, int PRW, int PSW, bool MAT, int SU>
+static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* ctas_out) {
+  constexpr bool SR = SU > 0;
+  auto kern = k_build_probe<KW, PRW, PSW, MAT, SU>;
+  JoinArgs a = a_in;
+  static const int nrb_env = env_int("HAPE_JN_NRB", 0), nsb_env = env_int("HAPE_JN_NSB", 0);
+  a.nsb = SR ? (uint32_t)std::min(8, std::max(2, nsb_env ? nsb_env : (SU >= 4 ? 3 : 2))) : 0u;
+  a.nrb = SR ? (uint32_t)std::min(2, std::max(1, nrb_env ? nrb_env : 2)) : 2u;
   static bool attr_set = false;
   if (!attr_set) {
     CK(h, cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024));
     attr_set = true;
   }
+  auto occ = [&](uint32_t sb, uint32_t nrb, int* per_sm) -> hape_status {
+    const size_t smem = join_smem_bytes<KW, PRW, PSW, SU>(a.cap, sb, nrb, a.nsb);
+    *per_sm = 0;
+    if (smem > 200 * 1024) return HAPE_OK;
+    CK(h, cudaOccupancyMaxActiveBlocksPerMultiprocessor(per_sm, kern, JN_THREADS, smem));
+    return HAPE_OK;
+  };
   int per_sm = 0;
-  CK(h, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, JN_THREADS, smem));
-  if (per_sm < 1) return fail(h, HAPE_ERR_UNSUPPORTED, "build+probe does not fit: smem %zu", smem);
+  CKS(occ(a.slot_bits, a.nrb, &per_sm));
+  // a single R buffer when the second one would cost a CTA per SM (SR: the
+  // other resident CTAs cover the R load at a stage boundary)
+  if (SR && !nrb_env && a.nrb == 2) {
+    int p1 = 0;
+    CKS(occ(a.slot_bits, 1, &p1));
+    if (p1 > per_sm) { a.nrb = 1; per_sm = p1; }
+  }
+  if (per_sm < 1)
+    return fail(h, HAPE_ERR_UNSUPPORTED, "build+probe does not fit: smem %zu",
+                join_smem_bytes<KW, PRW, PSW, SU>(a.cap, a.slot_bits, a.nrb, a.nsb));
   // plan.slot_bits is the minimum table size: one more bit (shorter chains)
   // when the larger head array costs no occupancy (register-limited kernels)
-  JoinArgs a2 = a;
   if (a.slot_bits < 14) {
-    const size_t smem2 = join_smem_bytes<KW, PRW>(a.cap, a.slot_bits + 1);
     int per_sm2 = 0;
-    CK(h, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm2, kern, JN_THREADS, smem2));
-    if (per_sm2 == per_sm) { a2.slot_bits = a.slot_bits + 1; }
+    CKS(occ(a.slot_bits + 1, a.nrb, &per_sm2));
+    if (per_sm2 == per_sm) a.slot_bits = a.slot_bits + 1;
   }
-  const size_t smem_used = join_smem_bytes<KW, PRW>(a2.cap, a2.slot_bits);
+  const size_t smem_used = join_smem_bytes<KW, PRW, PSW, SU>(a.cap, a.slot_bits, a.nrb, a.nsb);
   const unsigned grid = (unsigned)(per_sm * h->num_sms);
   *ctas_out = grid;
-  kern<<<grid, JN_THREADS, smem_used, h->stream>>>(a2);
+  kern<<<grid, JN_THREADS, smem_used, h->stream>>>(a);
   CK_LAUNCH(h);
   return HAPE_OK;
 }
 
 template <int KW, int PRW, int PSW>
 static hape_status launch_join_m(hape_join* h, const JoinArgs& a, bool mat, uint32_t* ctas) {
-  return mat ? launch_join_t<KW, PRW, PSW, true>(h, a, ctas) : launch_join_t<KW, PRW, PSW, false>(h, a, ctas);
+  // S tile tuples per thread of the SR form (0 = direct S loads)
+  static const int su_env = env_int("HAPE_JN_SU", -1);
+  const int su = su_env >= 0 ? su_env : ((mat || KW + PSW > 8) ? 4 : 0);  // measured best (C3: 14.1 -> 12.5 ms)
+#define HAPE_JN_SU(M)                                                  \
+  switch (su) {                                                        \
+    case 0: return launch_join_t<KW, PRW, PSW, M, 0>(h, a, ctas);      \
+    case 1: return launch_join_t<KW, PRW, PSW, M, 1>(h, a, ctas);      \
+    case 2: return launch_join_t<KW, PRW, PSW, M, 2>(h, a, ctas);      \
+    default: return launch_join_t<KW, PRW, PSW, M, 4>(h, a, ctas);     \
+  }
+  if (mat) { HAPE_JN_SU(true) } else { HAPE_JN_SU(false) }
+#undef HAPE_JN_SU
 }
 
 static hape_status launch_join(hape_join* h, int kw, int prw, int psw, const JoinArgs& a, bool mat,
@@ -715,6 +761,14 @@ static hape_status exchange(hape_join* h, Src in[2], Src out[2]) {
   const size_t nb = (size_t)G * 2 * (G + 1);
   if (h->h_bounds_cap < nb) {
     if (h->h_bounds) cudaFreeHost(h->h_bounds);
+  for (auto& p : h->hp)
+    if (p) cudaFreeHost(p);
+  for (auto& set : h->cpst)
+    for (auto& b : set)
+      if (b.p) cudaFree(b.p);
+  for (auto& pr : h->ev_h2d)
+    for (auto& e : pr)
+      if (e) cudaEventDestroy(e);
     CK(h, cudaMallocHost(&h->h_bounds, nb * 4));
     h->h_bounds_cap = nb;
   }
@@ -865,7 +919,7 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
     return HAPE_OK;
   };
   static const bool no_graph = getenv("HAPE_NO_GRAPH") != nullptr;
-  const bool graphable = !no_graph && world == 1 && !h->comm && R->mem == HAPE_MEM_DEVICE &&
+  const bool graphable = !no_graph && !h->in_coprocess && world == 1 && !h->comm && R->mem == HAPE_MEM_DEVICE &&
                          S->mem == HAPE_MEM_DEVICE && (!mat || out->mem == HAPE_MEM_DEVICE);
   if (graphable) {
     const uintptr_t key[] = {(uintptr_t)R->key, (uintptr_t)R->payload, (uintptr_t)R->n, (uintptr_t)S->key,
@@ -939,6 +993,8 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
 // ---------------------------------------------------------------------------
 // the non-partitioned GPU hash join (Fig. 6's baseline; nonpart.cuh)
 // ---------------------------------------------------------------------------
+#include "coprocess.cuh"
+
 template <int KW, int PRW, int PSW>
 static hape_status np_launch(hape_join* h, const Src& r, const Src& s, void* table, uint32_t mask, bool mat,
                              void* mat_r, void* mat_s, unsigned long long cap, unsigned long long* acc,
@@ -1059,7 +1115,7 @@ static hape_status np_join_impl(hape_join* h, const hape_relation* R, const hape
 // ---------------------------------------------------------------------------
 extern "C" {
 
-const char* hape_version(void) { return "hape-b200 1.1 (sm_100a, ABI 2)"; }
+const char* hape_version(void) { return "hape-b200 1.2 (sm_100a, ABI 3)"; }
 
 const char* hape_status_string(hape_status s) {
   switch (s) {
@@ -1116,6 +1172,10 @@ hape_status hape_join_create(const hape_join_config* cfg, hape_join** out_handle
     if (cudaStreamCreateWithFlags(&h->copy_stream, cudaStreamNonBlocking) != cudaSuccess ||
         cudaEventCreateWithFlags(&h->ev_copy, cudaEventDisableTiming) != cudaSuccess) { st = HAPE_ERR_CUDA; break; }
     if (st != HAPE_OK) break;
+    for (auto& pr : h->ev_h2d)
+      for (auto& e : pr)
+        if (cudaEventCreate(&e) != cudaSuccess) st = HAPE_ERR_CUDA;
+    if (st != HAPE_OK) break;
     if (cudaMallocHost(&h->h_res, 16 * sizeof(unsigned long long)) != cudaSuccess) { st = HAPE_ERR_OOM; break; }
     if (cfg->max_r || cfg->max_s) {
       hape_plan pl;
@@ -1132,6 +1192,31 @@ hape_status hape_join_create(const hape_join_config* cfg, hape_join** out_handle
   }
   *out_handle = h;
   return HAPE_OK;
+}
+
+hape_status hape_coprocess_join(hape_join* h, const hape_relation* R, const hape_relation* S,
+                                const hape_coprocess_config* cp, const hape_output* out, hape_join_result* res) {
+  if (!h) return HAPE_ERR_INVALID_ARG;
+  if (!res) return fail(h, HAPE_ERR_INVALID_ARG, "res is NULL");
+  try {
+    const hape_status st = coprocess_impl(h, R, S, cp, out, res);
+    h->in_coprocess = false;
+    return st;
+  } catch (...) {
+    h->in_coprocess = false;
+    return fail(h, HAPE_ERR_CUDA, "unexpected C++ exception (host partitioning threads)");
+  }
+}
+
+hape_status hape_host_partition(const hape_relation* rel, hape_dtype key_type, hape_dtype payload_type,
+                                hape_part_fn part_fn, uint32_t fanout_bits, int threads, void* out_keys,
+                                void* out_payloads, uint64_t* out_bounds) {
+  try {
+    return host_partition(rel, key_type, payload_type, part_fn, fanout_bits, threads, out_keys, out_payloads,
+                          out_bounds);
+  } catch (...) {
+    return HAPE_ERR_INVALID_ARG;
+  }
 }
 
 hape_status hape_join_destroy(hape_join* h) {
@@ -1151,6 +1236,14 @@ hape_status hape_join_destroy(hape_join* h) {
   if (h->np_table.p) cudaFree(h->np_table.p);
   if (h->h_res) cudaFreeHost(h->h_res);
   if (h->h_bounds) cudaFreeHost(h->h_bounds);
+  for (auto& p : h->hp)
+    if (p) cudaFreeHost(p);
+  for (auto& set : h->cpst)
+    for (auto& b : set)
+      if (b.p) cudaFree(b.p);
+  for (auto& pr : h->ev_h2d)
+    for (auto& e : pr)
+      if (e) cudaEventDestroy(e);
   for (auto& e : h->ev)
     if (e) cudaEventDestroy(e);
   if (h->copy_stream) { cudaStreamSynchronize(h->copy_stream); cudaStreamDestroy(h->copy_stream); }

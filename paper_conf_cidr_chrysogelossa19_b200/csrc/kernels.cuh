@@ -871,9 +871,23 @@ constexpr uint32_t JN_MAXCAP = 16384;
 constexpr uint32_t JN_NIL = 0xFFFFu;
 constexpr uint32_t JN_STOP = 0xFFFFFFFFu;
 
+
 template <int KW, int PRW>
-__host__ __device__ constexpr size_t join_smem_bytes(uint32_t cap, uint32_t slot_bits) {
-  return 2 * (((size_t)cap * sizeof(Tup<KW, PRW>) + 32 + 15) / 16 * 16)  // R ring
+__host__ __device__ constexpr size_t join_ring_bytes(uint32_t cap) {
+  return ((size_t)cap * sizeof(Tup<KW, PRW>) + 32 + 15) / 16 * 16;
+}
+// staged S tile: SU tuples per consumer thread
+template <int KW, int PSW, int SU>
+__host__ __device__ constexpr size_t join_stile_bytes() {
+  return ((size_t)SU * JN_CONSUMERS * sizeof(Tup<KW, PSW>) + 32 + 15) / 16 * 16;
+}
+// nrb R-chunk buffers, nsb staged S tiles of SU*256 tuples (SU = 0: S read
+// straight from HBM)
+template <int KW, int PRW, int PSW, int SU = 0>
+__host__ __device__ constexpr size_t join_smem_bytes(uint32_t cap, uint32_t slot_bits, uint32_t nrb = 2,
+                                                     uint32_t nsb = 0) {
+  return nrb * join_ring_bytes<KW, PRW>(cap)                               // R ring
+         + (SU ? nsb * join_stile_bytes<KW, PSW, SU>() : 0)               // S ring
          + ((size_t)cap * 2 + 15) / 16 * 16                                // next[]
          + ((size_t)4 << slot_bits);                                       // heads[]
 }
@@ -888,6 +902,8 @@ struct JoinArgs {
   uint32_t dbg;                              // timing experiments only (HAPE_JN_DBG); 0 in production
   uint32_t r_unique;                         // caller guarantees unique R keys (HAPE_FLAG_R_UNIQUE)
   uint32_t pf_bytes;                         // L2 prefetch window at the head of each S slice (0 = off)
+  uint32_t nrb;                              // R-chunk ring buffers (1 or 2)
+  uint32_t nsb;                              // SR kernels: staged S tiles in the ring (>= 2)
 };
 
 struct JnStage {
@@ -1037,17 +1053,32 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
   }
 }
 
-template <int KW, int PRW, int PSW, bool MAT>
+// SU > 0: the producer warp also stages the S slice through an nsb-deep
+// ring of SU*256-tuple tiles (bulk copies, mbarrier full/empty pairs; each
+// consumer warp releases a tile once its tuples are in registers), so the
+// consumers never wait on HBM latency -- the form for materialising and
+// 16-byte-tuple joins, whose probe cannot keep a software-pipelined S batch
+// in registers.
+template <int KW, int PRW, int PSW, bool MAT, int SU>
 __global__ void __launch_bounds__(JN_THREADS)
 k_build_probe(JoinArgs a) {
+  constexpr bool SR = SU > 0;
+  constexpr uint32_t JN_STILE = (uint32_t)(SR ? SU : 1) * JN_CONSUMERS;
   using TR = Tup<KW, PRW>;
+  using TS = Tup<KW, PSW>;
   extern __shared__ __align__(128) unsigned char smem[];
-  const uint32_t RB = ((uint32_t)(a.cap * sizeof(TR)) + 32 + 15) / 16 * 16;
-  unsigned char* ring = smem;                                           // [2][RB]
-  uint16_t* s_next = reinterpret_cast<uint16_t*>(smem + 2 * RB);
-  uint32_t* s_head = reinterpret_cast<uint32_t*>(smem + 2 * RB + ((size_t)a.cap * 2 + 15) / 16 * 16);
+  const uint32_t RB = (uint32_t)join_ring_bytes<KW, PRW>(a.cap);
+  constexpr uint32_t SB = SR ? (uint32_t)join_stile_bytes<KW, PSW, SR ? SU : 1>() : 0u;
+  const uint32_t NRB = SR ? a.nrb : 2u, NSB = SR ? a.nsb : 0u;
+  unsigned char* ring = smem;                                           // [NRB][RB]
+  unsigned char* sring = smem + NRB * RB;                               // [NSB][SB]
+  uint16_t* s_next = reinterpret_cast<uint16_t*>(sring + NSB * SB);
+  uint32_t* s_head = reinterpret_cast<uint32_t*>(reinterpret_cast<unsigned char*>(s_next) +
+                                                 ((size_t)a.cap * 2 + 15) / 16 * 16);
+  constexpr int MAXS = 8;
   __shared__ JnStage s_meta[2];
-  __shared__ __align__(8) uint64_t full[2], empty[2];
+  __shared__ uint32_t s_soff[MAXS];
+  __shared__ __align__(8) uint64_t full[2], empty[2], sfull[MAXS], sempty[MAXS];
   __shared__ uint32_t s_wsum[JN_CONSUMERS / 32];
   __shared__ unsigned long long s_wbase[JN_CONSUMERS / 32];
   __shared__ unsigned long long s_red[4][JN_THREADS / 32];
@@ -1057,7 +1088,8 @@ k_build_probe(JoinArgs a) {
   JnAcc acc;
 
   if (threadIdx.x == 0) {
-    for (int i = 0; i < 2; i++) { mbar_init(&full[i], 1); mbar_init(&empty[i], 1); }
+    for (uint32_t i = 0; i < NRB; i++) { mbar_init(&full[i], 1); mbar_init(&empty[i], 1); }
+    for (uint32_t i = 0; i < NSB; i++) { mbar_init(&sfull[i], 1); mbar_init(&sempty[i], JN_CONSUMERS / 32); }
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
   }
   __syncthreads();
@@ -1068,9 +1100,8 @@ k_build_probe(JoinArgs a) {
       const uint64_t pol = policy_evict_first();
       const uint32_t n_items = *a.n_items;
       const TR* rT = static_cast<const TR*>(a.rt);
-      using TS = Tup<KW, PSW>;
       const TS* sT = static_cast<const TS*>(a.st);
-      uint32_t stage = 0;
+      uint32_t stage = 0, sseq = 0;
       for (uint32_t it = blockIdx.x; it < n_items; it += gridDim.x) {
         const uint2 item = a.items[it];
         const uint32_t q = item.x;
@@ -1078,7 +1109,7 @@ k_build_probe(JoinArgs a) {
         const uint32_t s_lo = a.bS[q] + item.y * a.slice;
         const uint32_t s_hi = min(a.bS[q + 1], s_lo + a.slice);
         for (uint32_t c_lo = r_lo; c_lo < r_hi; c_lo += a.cap, stage++) {
-          const uint32_t bi = stage & 1, ph = (stage >> 1) & 1;
+          const uint32_t bi = stage % NRB, ph = (stage / NRB) & 1;
           mbar_wait_backoff(&empty[bi], ph ^ 1);
           const uint32_t nr = min(a.cap, r_hi - c_lo);
           const uintptr_t ra = reinterpret_cast<uintptr_t>(rT + c_lo);
@@ -1086,20 +1117,35 @@ k_build_probe(JoinArgs a) {
           s_meta[bi] = JnStage{nr, (uint32_t)(ra - r0), s_lo, s_hi};
           mbar_expect_tx(&full[bi], (uint32_t)(r1 - r0));
           bulk_g2s(ring + bi * RB, reinterpret_cast<const void*>(r0), (uint32_t)(r1 - r0), &full[bi], pol);
-          // warm L2 with the stage's S slice: the consumers reach it a stage later
-          if (c_lo == r_lo && s_hi > s_lo && a.pf_bytes)
-            bulk_prefetch_l2(sT + s_lo, min((size_t)(s_hi - s_lo) * sizeof(TS), (size_t)a.pf_bytes));
+          if constexpr (SR) {
+            // the stage's S slice, tile by tile, through the S ring
+            for (uint32_t t0 = s_lo; t0 < s_hi; t0 += JN_STILE, sseq++) {
+              const uint32_t sb = sseq % NSB, sph = (sseq / NSB) & 1;
+              mbar_wait_backoff(&sempty[sb], sph ^ 1);
+              const uint32_t n = min(JN_STILE, s_hi - t0);
+              const uintptr_t sa = reinterpret_cast<uintptr_t>(sT + t0);
+              const uintptr_t a0 = sa & ~(uintptr_t)15, a1 = (sa + (size_t)n * sizeof(TS) + 15) & ~(uintptr_t)15;
+              s_soff[sb] = (uint32_t)(sa - a0);
+              mbar_expect_tx(&sfull[sb], (uint32_t)(a1 - a0));
+              bulk_g2s(sring + sb * SB, reinterpret_cast<const void*>(a0), (uint32_t)(a1 - a0), &sfull[sb], pol);
+            }
+          } else {
+            // warm L2 with the stage's S slice: the consumers reach it a stage later
+            if (c_lo == r_lo && s_hi > s_lo && a.pf_bytes)
+              bulk_prefetch_l2(sT + s_lo, min((size_t)(s_hi - s_lo) * sizeof(TS), (size_t)a.pf_bytes));
+          }
         }
       }
-      const uint32_t bi = stage & 1, ph = (stage >> 1) & 1;
+      const uint32_t bi = stage % NRB, ph = (stage / NRB) & 1;
       mbar_wait_backoff(&empty[bi], ph ^ 1);
       s_meta[bi].nr = JN_STOP;
       mbar_arrive(&full[bi]);
     }
   } else {
     // ------------------------------ consumer warps -----------------------------
+    uint32_t sseq = 0;
     for (uint32_t stage = 0;; stage++) {
-      const uint32_t bi = stage & 1, ph = (stage >> 1) & 1;
+      const uint32_t bi = stage % NRB, ph = (stage / NRB) & 1;
       // reset the heads (the previous stage's probe is complete: see the
       // barrier at the end of the loop body), then wait for the R chunk
       for (uint32_t i = threadIdx.x * 4; i < nslots; i += JN_CONSUMERS * 4)
@@ -1116,7 +1162,7 @@ k_build_probe(JoinArgs a) {
       // (materialising kernels hold more live state: there the batch is
       // loaded just before it is probed -- HAPE measured the pipelined form 2x
       // slower for C3)
-      constexpr bool PIPE = !MAT;
+      constexpr bool PIPE = !MAT && !SR;
       Tup<KW, PSW> xs[JN_U];
       if (PIPE && st.s_lo + BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U>(a, st.s_lo, st.s_hi, xs);
       if (!(a.dbg & 4u))
@@ -1125,35 +1171,57 @@ k_build_probe(JoinArgs a) {
       consumer_sync();
       // ---- probe (a12): stream the S slice.  Bag semantics walk every chain
       // to its end; a caller-declared unique build side (HAPE_FLAG_R_UNIQUE, a
-      // primary key) stops at the first match.  Full batches are software
-      // pipelined: batch b+1 is loaded into registers while b is probed.
+      // primary key) stops at the first match.
       const JnTable<KW, PRW> tab{r, s_next, s_head, a.slot_bits, a.r_unique == 0};
-      uint32_t base = st.s_lo;
-      while (base + BATCH <= st.s_hi) {
-        Tup<KW, PSW> x[JN_U];
-        if constexpr (PIPE) {
+      if constexpr (SR) {
+        // staged S tiles: wait for the tile, copy this thread's tuples to
+        // registers, release the tile (one arrival per warp), probe
+        for (uint32_t base = st.s_lo; base < st.s_hi; base += JN_STILE, sseq++) {
+          const uint32_t sb = sseq % NSB, sph = (sseq / NSB) & 1;
+          mbar_wait(&sfull[sb], sph);
+          const TS* tile = reinterpret_cast<const TS*>(sring + sb * SB + s_soff[sb]);
+          const uint32_t n = min(JN_STILE, st.s_hi - base);
+          constexpr int XU = SR ? SU : 1;
+          Tup<KW, PSW> x[XU];
 #pragma unroll
-          for (int u = 0; u < JN_U; u++) x[u] = xs[u];
-          if (base + 2 * BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U>(a, base + BATCH, st.s_hi, xs);
-        } else {
-          jn_load_batch<KW, PSW, JN_U>(a, base, st.s_hi, x);
+          for (int u = 0; u < XU; u++) {
+            const uint32_t j = u * JN_CONSUMERS + threadIdx.x;
+            if (j < n) x[u] = tile[j];
+          }
+          __syncwarp();
+          if (lane == 0) mbar_arrive(&sempty[sb]);
+          jn_probe_batch<KW, PRW, PSW, MAT, XU>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
         }
-        jn_probe_batch<KW, PRW, PSW, MAT, JN_U>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
-        base += BATCH;
-      }
-      const uint32_t rem = st.s_hi > base ? st.s_hi - base : 0;
-      if (rem > 2 * JN_CONSUMERS) {
-        Tup<KW, PSW> x[4];
-        jn_load_batch<KW, PSW, 4>(a, base, st.s_hi, x);
-        jn_probe_batch<KW, PRW, PSW, MAT, 4>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
-      } else if (rem > JN_CONSUMERS) {
-        Tup<KW, PSW> x[2];
-        jn_load_batch<KW, PSW, 2>(a, base, st.s_hi, x);
-        jn_probe_batch<KW, PRW, PSW, MAT, 2>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
-      } else if (rem > 0) {
-        Tup<KW, PSW> x[1];
-        jn_load_batch<KW, PSW, 1>(a, base, st.s_hi, x);
-        jn_probe_batch<KW, PRW, PSW, MAT, 1>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+      } else {
+        // Full batches are software pipelined (PIPE): batch b+1 is loaded into
+        // registers while b is probed.
+        uint32_t base = st.s_lo;
+        while (base + BATCH <= st.s_hi) {
+          Tup<KW, PSW> x[JN_U];
+          if constexpr (PIPE) {
+#pragma unroll
+            for (int u = 0; u < JN_U; u++) x[u] = xs[u];
+            if (base + 2 * BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U>(a, base + BATCH, st.s_hi, xs);
+          } else {
+            jn_load_batch<KW, PSW, JN_U>(a, base, st.s_hi, x);
+          }
+          jn_probe_batch<KW, PRW, PSW, MAT, JN_U>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+          base += BATCH;
+        }
+        const uint32_t rem = st.s_hi > base ? st.s_hi - base : 0;
+        if (rem > 2 * JN_CONSUMERS) {
+          Tup<KW, PSW> x[4];
+          jn_load_batch<KW, PSW, 4>(a, base, st.s_hi, x);
+          jn_probe_batch<KW, PRW, PSW, MAT, 4>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+        } else if (rem > JN_CONSUMERS) {
+          Tup<KW, PSW> x[2];
+          jn_load_batch<KW, PSW, 2>(a, base, st.s_hi, x);
+          jn_probe_batch<KW, PRW, PSW, MAT, 2>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+        } else if (rem > 0) {
+          Tup<KW, PSW> x[1];
+          jn_load_batch<KW, PSW, 1>(a, base, st.s_hi, x);
+          jn_probe_batch<KW, PRW, PSW, MAT, 1>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+        }
       }
       consumer_sync();  // everyone is done with heads/next and ring buffer bi
       if (threadIdx.x == 0) mbar_arrive(&empty[bi]);
