@@ -70,3 +70,38 @@ def test_host_partition_rejects_bad_args():
 def test_coprocess_rejects_without_gpu_work():
     """Argument errors surface before any device work (NULL handle / result)."""
     assert _lib.lib.hape_coprocess_join(None, None, None, None, None, None) == _lib.HAPE_ERR_INVALID_ARG
+
+
+@pytest.mark.parametrize("shift", [1, 3, 5])
+def test_host_partition_unaligned_outputs(shift):
+    """Output columns that do not start on a 64-byte line (the write-combining
+    path's slot arithmetic) give the same stable partition."""
+    rng = np.random.default_rng(shift)
+    n = 100_001
+    k = rng.integers(-2**31, 2**31, size=n).astype(np.int32)
+    p = rng.integers(-2**40, 2**40, size=n).astype(np.int64)
+    ok = np.zeros(n + 16, np.int32)
+    op = np.zeros(n + 16, np.int64)
+    rel = _lib.hape_relation(k.ctypes.data, p.ctypes.data, n, _lib.HAPE_MEM_HOST)
+    b = (ctypes.c_uint64 * 9)()
+    st = _lib.hape_host_partition(rel, _lib.HAPE_INT32, _lib.HAPE_INT64, _lib.HAPE_PART_HASH, 3, 6,
+                                  ok.ctypes.data + 4 * shift, op.ctypes.data + 8 * shift, b)
+    assert st == _lib.HAPE_OK
+    ek, ep, eb = _expected(k, p, 3)
+    assert np.array_equal(ok[shift:shift + n], ek) and np.array_equal(op[shift:shift + n], ep)
+    assert not ok[:shift].any() and not ok[shift + n:].any() and not op[shift + n:].any()
+    assert np.array_equal(np.array(list(b)), eb)
+
+
+@pytest.mark.parametrize("n", [1, 3, 9, 40])
+def test_host_partition_unaligned_tiny(n):
+    k = np.arange(n, dtype=np.int64) * 977 - 5
+    p = np.arange(n, dtype=np.int64)
+    ok = np.zeros(n + 8, np.int64)
+    op = np.zeros(n + 8, np.int64)
+    rel = _lib.hape_relation(k.ctypes.data, p.ctypes.data, n, _lib.HAPE_MEM_HOST)
+    b = (ctypes.c_uint64 * 5)()
+    assert _lib.hape_host_partition(rel, _lib.HAPE_INT64, _lib.HAPE_INT64, _lib.HAPE_PART_HASH, 2, 2,
+                                    ok.ctypes.data + 40, op.ctypes.data + 24, b) == _lib.HAPE_OK
+    ek, ep, _ = _expected(k, p, 2)
+    assert np.array_equal(ok[5:5 + n], ek) and np.array_equal(op[3:3 + n], ep)
