@@ -1172,10 +1172,6 @@ hape_status hape_join_create(const hape_join_config* cfg, hape_join** out_handle
     if (cudaStreamCreateWithFlags(&h->copy_stream, cudaStreamNonBlocking) != cudaSuccess ||
         cudaEventCreateWithFlags(&h->ev_copy, cudaEventDisableTiming) != cudaSuccess) { st = HAPE_ERR_CUDA; break; }
     if (st != HAPE_OK) break;
-    for (auto& pr : h->ev_h2d)
-      for (auto& e : pr)
-        if (cudaEventCreate(&e) != cudaSuccess) st = HAPE_ERR_CUDA;
-    if (st != HAPE_OK) break;
     if (cudaMallocHost(&h->h_res, 16 * sizeof(unsigned long long)) != cudaSuccess) { st = HAPE_ERR_OOM; break; }
     if (cfg->max_r || cfg->max_s) {
       hape_plan pl;
