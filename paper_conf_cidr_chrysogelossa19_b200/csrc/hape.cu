@@ -226,7 +226,7 @@ static hape_status make_plan(const hape_join* h, uint64_t n_r, uint64_t n_s, hap
     const int sbi = (int)ceil_log2_u64(std::min<uint64_t>(std::max<uint64_t>(expected, 1), cap)) + extra;
     sb = (uint32_t)std::max(6, std::min(sbi, 14));
     const size_t bytes = 2 * ((cap * kwb + 47) / 16 * 16 + (cap * prw + 47) / 16 * 16) + (cap * 2 + 15) / 16 * 16 +
-                         ((size_t)4 << sb);
+                         (sizeof(JnHead) << sb);
     if (bytes <= 110 * 1024 || cap <= 256) break;
     cap -= 128;
   }
@@ -454,10 +454,11 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
                 join_smem_bytes<KW, PRW, PSW, SU>(a.cap, a.slot_bits, a.nrb, a.nsb));
   // plan.slot_bits is the minimum table size: one more bit (shorter chains)
   // when the larger head array costs no occupancy (register-limited kernels)
-  if (a.slot_bits < 14) {
+  while (a.slot_bits < 14) {
     int per_sm2 = 0;
     CKS(occ(a.slot_bits + 1, a.nrb, &per_sm2));
-    if (per_sm2 == per_sm) a.slot_bits = a.slot_bits + 1;
+    if (per_sm2 != per_sm) break;
+    a.slot_bits = a.slot_bits + 1;
   }
   const size_t smem_used = join_smem_bytes<KW, PRW, PSW, SU>(a.cap, a.slot_bits, a.nrb, a.nsb);
   const unsigned grid = (unsigned)(per_sm * h->num_sms);
