@@ -350,9 +350,39 @@ def main():
         barrier()
         e_ms = max_over_ranks(e0.elapsed_time(e1) / n_e2e)
         h2d = sum(x.numel() * x.element_size() for x in hk)
+        # host-link roofline of the e2e step: a plain pinned H2D copy of the
+        # same byte count, timed here with CUDA events (no join work)
+        pcie = None
+        try:
+            src = hk[0] if hk[0].numel() * hk[0].element_size() >= (256 << 20) else None
+            if src is not None:
+                dst = torch.empty(src.shape, dtype=src.dtype, device="cuda")
+                for _ in range(2):
+                    dst.copy_(src, non_blocking=True)
+                torch.cuda.synchronize()
+                e0.record(stream)
+                for _ in range(3):
+                    dst.copy_(src, non_blocking=True)
+                e1.record(stream)
+                torch.cuda.synchronize()
+                bw = 3 * src.numel() * src.element_size() / (e0.elapsed_time(e1) / 1000.0)
+                e0.record(stream)
+                for _ in range(3):
+                    src.copy_(dst, non_blocking=True)
+                e1.record(stream)
+                torch.cuda.synchronize()
+                bw_d = 3 * src.numel() * src.element_size() / (e0.elapsed_time(e1) / 1000.0)
+                del dst
+                d2h_b = d2h // n_e2e
+                # the call moves its inputs in and its result (and pairs) out in sequence
+                bound = (h2d / bw + d2h_b / bw_d) * 1000.0
+                pcie = {"h2d_GB/s_measured": round(bw / 1e9, 1), "d2h_GB/s_measured": round(bw_d / 1e9, 1),
+                        "bound_ms": round(bound, 3), "frac": round(bound / e_ms, 3)}
+        except Exception as ex:
+            pcie = {"error": repr(ex)}
         e2e = {"value": total_tuples / (e_ms / 1000.0), "unit": UNIT, "ms_per_step": e_ms,
                "h2d_bytes_per_step": h2d, "d2h_bytes_per_step": d2h // n_e2e,
-               "h2d_stage_ms": r2.stage_ms.get("h2d")}
+               "h2d_stage_ms": r2.stage_ms.get("h2d"), "pcie_roofline": pcie}
         # ---- PAPER.md §5 / Fig. 7 co-processing on the same host-resident
         # inputs: CPU-side co-partitioning into F pairs, one transfer per pair
         # overlapping the previous pair's device join (hape_coprocess_join,
