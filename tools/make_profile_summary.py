@@ -67,9 +67,14 @@ def full_metrics(path):
 
 L = launches()
 items = list(L.items())
-# the profiled step = launches after the last 3 warm-up steps: take the tail
-per_step = {"c1": 8, "c2": 14, "c3": 14}.get(CFG, 14)
-step = items[-per_step:]
+# the profiled step = the launches after the previous step's build+probe up
+# to the last build+probe (ablation kernels after it are not part of a step)
+bps = [k for k, ((i, n, g, b), m) in enumerate(items) if "k_build_probe" in n]
+if len(bps) >= 2:
+    step = items[bps[-2] + 1: bps[-1] + 1]
+else:
+    per_step = {"c1": 8, "c2": 14, "c3": 14}.get(CFG, 14)
+    step = items[-per_step:]
 lines = [f"# ncu summary {TAG} / {CFG}\n",
          "Per-launch list of ONE bench step (`ncu --metrics gpu__time_duration.sum,dram__bytes_read.sum,"
          "dram__bytes_write.sum --clock-control none`): cold-cache, serialised launches -- compare shares, "
@@ -85,7 +90,7 @@ traffic = {}
 lines.append("## --set full captures (per launch)\n")
 lines.append("| kernel | us | DRAM rd+wr MB | TB/s | warp inst M | IPC | occ % | regs | smem wavefronts M | L1 % | DRAM % | top stalls |")
 lines.append("|---|---|---|---|---|---|---|---|---|---|---|---|")
-for name in ("k_hist", "k_scatter", "k_build_probe"):
+for name in ("k_hist", "k_hist_joint", "k_scatter", "k_build_probe"):
     path = os.path.join(G, f"full_{TAG}_{CFG}_{name}.ncu-rep")
     if not os.path.exists(path):
         continue

@@ -8,7 +8,7 @@ nvidia-smi --query-gpu=index,clocks.sm,clocks.max.sm,power.draw,clocks_event_rea
 SMI=$!
 timeout 600 python bench.py --config $CFG > gpurun_out/bench_${TAG}_${CFG}.json 2> gpurun_out/bench_${TAG}_${CFG}.err
 kill $SMI
-B="python bench.py --config $CFG --steps 1 --warmup 3 --no-e2e --no-cpu-baseline"
+B="python bench.py --config $CFG --steps 1 --warmup 3 --no-e2e --no-cpu-baseline --no-ablation --no-coprocess"
 timeout 600 ncu --metrics gpu__time_duration.sum,dram__bytes_read.sum,dram__bytes_write.sum --clock-control none --csv --log-file gpurun_out/launches_${TAG}_${CFG}.csv $B > /dev/null 2>&1
 # per-launch skip counts: 3 warm-up steps precede the profiled one
 # (two-pass plans: one joint histogram per relation and step, 4 scatters)
