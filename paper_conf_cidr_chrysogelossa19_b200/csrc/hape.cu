@@ -420,10 +420,11 @@ static int env_int(const char* name, int dflt) {
   return e ? atoi(e) : dflt;
 }
 
-template <int KW, int PRW, int PSW, bool MAT, int SU>
+template <int KW, int PRW, int PSW, bool MAT, int SU, int NC = 256>
 static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* ctas_out) {
   constexpr bool SR = SU > 0;
-  auto kern = k_build_probe<KW, PRW, PSW, MAT, SU>;
+  constexpr int JN_THREADS = NC + 32;
+  auto kern = k_build_probe<KW, PRW, PSW, MAT, SU, NC>;
   JoinArgs a = a_in;
   static const int nrb_env = env_int("HAPE_JN_NRB", 0), nsb_env = env_int("HAPE_JN_NSB", 0);
   a.nsb = SR ? (uint32_t)std::min(8, std::max(2, nsb_env ? nsb_env : (SU >= 4 ? 3 : 2))) : 0u;
@@ -434,7 +435,7 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
     attr_set = true;
   }
   auto occ = [&](uint32_t sb, uint32_t nrb, int* per_sm) -> hape_status {
-    const size_t smem = join_smem_bytes<KW, PRW, PSW, SU>(a.cap, sb, nrb, a.nsb);
+    const size_t smem = join_smem_bytes<KW, PRW, PSW, SU, NC>(a.cap, sb, nrb, a.nsb);
     *per_sm = 0;
     if (smem > 200 * 1024) return HAPE_OK;
     CK(h, cudaOccupancyMaxActiveBlocksPerMultiprocessor(per_sm, kern, JN_THREADS, smem));
@@ -451,7 +452,7 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
   }
   if (per_sm < 1)
     return fail(h, HAPE_ERR_UNSUPPORTED, "build+probe does not fit: smem %zu",
-                join_smem_bytes<KW, PRW, PSW, SU>(a.cap, a.slot_bits, a.nrb, a.nsb));
+                join_smem_bytes<KW, PRW, PSW, SU, NC>(a.cap, a.slot_bits, a.nrb, a.nsb));
   // plan.slot_bits is the minimum table size: one more bit (shorter chains)
   // when the larger head array costs no occupancy (register-limited kernels)
   while (a.slot_bits < 14) {
@@ -460,7 +461,7 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
     if (per_sm2 != per_sm) break;
     a.slot_bits = a.slot_bits + 1;
   }
-  const size_t smem_used = join_smem_bytes<KW, PRW, PSW, SU>(a.cap, a.slot_bits, a.nrb, a.nsb);
+  const size_t smem_used = join_smem_bytes<KW, PRW, PSW, SU, NC>(a.cap, a.slot_bits, a.nrb, a.nsb);
   const unsigned grid = (unsigned)(per_sm * h->num_sms);
   *ctas_out = grid;
   kern<<<grid, JN_THREADS, smem_used, h->stream>>>(a);
@@ -470,17 +471,26 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
 
 template <int KW, int PRW, int PSW>
 static hape_status launch_join_m(hape_join* h, const JoinArgs& a, bool mat, uint32_t* ctas) {
-  // S tile tuples per thread of the SR form (0 = direct S loads)
-  static const int su_env = env_int("HAPE_JN_SU", -1);
-  const int su = su_env >= 0 ? su_env : ((mat || KW + PSW > 8) ? 4 : 0);  // measured best (C3: 14.1 -> 12.5 ms)
-#define HAPE_JN_SU(M)                                                  \
-  switch (su) {                                                        \
-    case 0: return launch_join_t<KW, PRW, PSW, M, 0>(h, a, ctas);      \
-    case 1: return launch_join_t<KW, PRW, PSW, M, 1>(h, a, ctas);      \
-    case 2: return launch_join_t<KW, PRW, PSW, M, 2>(h, a, ctas);      \
-    default: return launch_join_t<KW, PRW, PSW, M, 4>(h, a, ctas);     \
+  // S tile tuples per thread of the SR form (0 = direct S loads); consumer
+  // threads per CTA (HAPE_JN_NC=512: twice the warps per CTA)
+  // Measured (C3 build+probe): direct 14.1 ms; SR 256 threads, 1024-tuple
+  // tiles 12.4; SR 512 threads, 1024-tuple tiles 10.7 ms.  C2 (8-byte tuples,
+  // no pairs): direct 256 threads 0.74 ms, every SR / 512-thread form slower.
+  static const int su_env = env_int("HAPE_JN_SU", -1), nc_env = env_int("HAPE_JN_NC", 0);
+  const bool sr_form = mat || KW + PSW > 8;
+  const int su = su_env >= 0 ? su_env : (sr_form ? 2 : 0);
+  const bool wide = nc_env ? nc_env == 512 : sr_form;
+#define HAPE_JN_SU(M, NC)                                                  \
+  switch (su) {                                                            \
+    case 0: return launch_join_t<KW, PRW, PSW, M, 0, NC>(h, a, ctas);      \
+    case 1: return launch_join_t<KW, PRW, PSW, M, 1, NC>(h, a, ctas);      \
+    case 2: return launch_join_t<KW, PRW, PSW, M, 2, NC>(h, a, ctas);      \
+    default: return launch_join_t<KW, PRW, PSW, M, 4, NC>(h, a, ctas);     \
   }
-  if (mat) { HAPE_JN_SU(true) } else { HAPE_JN_SU(false) }
+  if (wide) {
+    if (mat) { HAPE_JN_SU(true, 512) } else { HAPE_JN_SU(false, 512) }
+  }
+  if (mat) { HAPE_JN_SU(true, 256) } else { HAPE_JN_SU(false, 256) }
 #undef HAPE_JN_SU
 }
 

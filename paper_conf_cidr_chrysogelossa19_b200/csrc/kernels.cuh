@@ -864,8 +864,8 @@ k_worklist(const uint32_t* __restrict__ bR, const uint32_t* __restrict__ bS, uin
 // the chain is walked to its end (bag semantics); the aggregation body of a
 // match runs with the lanes converged, once per round.
 // --------------------------------------------------------------------------
-constexpr int JN_CONSUMERS = 256;
-constexpr int JN_THREADS = JN_CONSUMERS + 32;
+// consumer threads per build+probe CTA: a template parameter (JN_CONSUMERS,
+// 256 or 512) of the kernel; one producer warp on top
 constexpr int JN_U = 4;
 constexpr uint32_t JN_MAXCAP = 16384;
 constexpr uint32_t JN_NIL = 0xFFFFu;
@@ -880,17 +880,17 @@ __host__ __device__ constexpr size_t join_ring_bytes(uint32_t cap) {
   return ((size_t)cap * sizeof(Tup<KW, PRW>) + 32 + 15) / 16 * 16;
 }
 // staged S tile: SU tuples per consumer thread
-template <int KW, int PSW, int SU>
+template <int KW, int PSW, int SU, int NC = 256>
 __host__ __device__ constexpr size_t join_stile_bytes() {
-  return ((size_t)SU * JN_CONSUMERS * sizeof(Tup<KW, PSW>) + 32 + 15) / 16 * 16;
+  return ((size_t)SU * NC * sizeof(Tup<KW, PSW>) + 32 + 15) / 16 * 16;
 }
 // nrb R-chunk buffers, nsb staged S tiles of SU*256 tuples (SU = 0: S read
 // straight from HBM)
-template <int KW, int PRW, int PSW, int SU = 0>
+template <int KW, int PRW, int PSW, int SU = 0, int NC = 256>
 __host__ __device__ constexpr size_t join_smem_bytes(uint32_t cap, uint32_t slot_bits, uint32_t nrb = 2,
                                                      uint32_t nsb = 0) {
   return nrb * join_ring_bytes<KW, PRW>(cap)                               // R ring
-         + (SU ? nsb * join_stile_bytes<KW, PSW, SU>() : 0)               // S ring
+         + (SU ? nsb * join_stile_bytes<KW, PSW, SU, NC>() : 0)           // S ring
          + ((size_t)cap * 2 + 15) / 16 * 16                                // next[]
          + (sizeof(JnHead) << slot_bits);                                  // heads[]
 }
@@ -915,8 +915,9 @@ struct JnStage {
   uint32_t s_lo, s_hi;
 };
 
+template <int NC>
 __device__ __forceinline__ void consumer_sync() {
-  asm volatile("bar.sync 1, %0;" ::"n"(JN_CONSUMERS) : "memory");
+  asm volatile("bar.sync 1, %0;" ::"n"(NC) : "memory");
 }
 
 // slot of a key in the smem table: top slot_bits bits of key * odd constant
@@ -940,7 +941,7 @@ struct JnTable {
 };
 
 // Load U S tuples per consumer thread: j = base + u*256 + tid.
-template <int KW, int PSW, int U>
+template <int KW, int PSW, int U, int JN_CONSUMERS>
 __device__ __forceinline__ void jn_load_batch(const JoinArgs& a, uint32_t base, uint32_t s_hi, Tup<KW, PSW> (&x)[U]) {
   const Tup<KW, PSW>* __restrict__ sT = static_cast<const Tup<KW, PSW>*>(a.st);
 #pragma unroll
@@ -951,7 +952,7 @@ __device__ __forceinline__ void jn_load_batch(const JoinArgs& a, uint32_t base, 
 }
 
 // Probe the U S tuples x[] (loaded by jn_load_batch for the same base).
-template <int KW, int PRW, int PSW, bool MAT, int U>
+template <int KW, int PRW, int PSW, bool MAT, int U, int JN_CONSUMERS>
 __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const JoinArgs& a, uint32_t base,
                                                uint32_t s_hi, const Tup<KW, PSW> (&x)[U], JnAcc& acc,
                                                uint32_t* s_wsum, unsigned long long* s_wbase) {
@@ -1015,7 +1016,7 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
       }
     }
     if (lane == 0) s_wsum[warp] = wtot;
-    consumer_sync();
+    consumer_sync<JN_CONSUMERS>();
     if (warp == 0) {
       const uint32_t v = lane < JN_CONSUMERS / 32 ? s_wsum[lane] : 0u;
       const uint32_t inc = warp_incl_scan(v);
@@ -1025,7 +1026,7 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
       g = __shfl_sync(0xffffffffu, g, 0);
       if (lane < JN_CONSUMERS / 32) s_wbase[lane] = g + inc - v;
     }
-    consumer_sync();
+    consumer_sync<JN_CONSUMERS>();
     const unsigned long long wb = s_wbase[warp];
     if (!t.dup) {
 #pragma unroll
@@ -1062,16 +1063,17 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
 // consumers never wait on HBM latency -- the form for materialising and
 // 16-byte-tuple joins, whose probe cannot keep a software-pipelined S batch
 // in registers.
-template <int KW, int PRW, int PSW, bool MAT, int SU>
-__global__ void __launch_bounds__(JN_THREADS)
+template <int KW, int PRW, int PSW, bool MAT, int SU, int JN_CONSUMERS = 256>
+__global__ void __launch_bounds__(JN_CONSUMERS + 32)
 k_build_probe(JoinArgs a) {
+  constexpr int JN_THREADS = JN_CONSUMERS + 32;
   constexpr bool SR = SU > 0;
   constexpr uint32_t JN_STILE = (uint32_t)(SR ? SU : 1) * JN_CONSUMERS;
   using TR = Tup<KW, PRW>;
   using TS = Tup<KW, PSW>;
   extern __shared__ __align__(128) unsigned char smem[];
   const uint32_t RB = (uint32_t)join_ring_bytes<KW, PRW>(a.cap);
-  constexpr uint32_t SB = SR ? (uint32_t)join_stile_bytes<KW, PSW, SR ? SU : 1>() : 0u;
+  constexpr uint32_t SB = SR ? (uint32_t)join_stile_bytes<KW, PSW, SR ? SU : 1, JN_CONSUMERS>() : 0u;
   const uint32_t NRB = SR ? a.nrb : 2u, NSB = SR ? a.nsb : 0u;
   unsigned char* ring = smem;                                           // [NRB][RB]
   unsigned char* sring = smem + NRB * RB;                               // [NSB][SB]
@@ -1161,7 +1163,7 @@ k_build_probe(JoinArgs a) {
       const JnStage st = s_meta[bi];
       if (st.nr == JN_STOP) break;
       const TR* r = reinterpret_cast<const TR*>(ring + bi * RB + st.off);
-      consumer_sync();
+      consumer_sync<JN_CONSUMERS>();
       // ---- build (a11): chained table via atomicExch on the heads
       // the first S batch is loaded before the build so its latency hides
       // behind the table construction
@@ -1171,11 +1173,11 @@ k_build_probe(JoinArgs a) {
       // slower for C3)
       constexpr bool PIPE = !MAT && !SR;
       Tup<KW, PSW> xs[JN_U];
-      if (PIPE && st.s_lo + BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U>(a, st.s_lo, st.s_hi, xs);
+      if (PIPE && st.s_lo + BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, st.s_lo, st.s_hi, xs);
       if (!(a.dbg & 4u))
         for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
           s_next[i] = (uint16_t)atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], i);
-      consumer_sync();
+      consumer_sync<JN_CONSUMERS>();
       // ---- probe (a12): stream the S slice.  Bag semantics walk every chain
       // to its end; a caller-declared unique build side (HAPE_FLAG_R_UNIQUE, a
       // primary key) stops at the first match.
@@ -1197,7 +1199,7 @@ k_build_probe(JoinArgs a) {
           }
           __syncwarp();
           if (lane == 0) mbar_arrive(&sempty[sb]);
-          jn_probe_batch<KW, PRW, PSW, MAT, XU>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+          jn_probe_batch<KW, PRW, PSW, MAT, XU, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
         }
       } else {
         // Full batches are software pipelined (PIPE): batch b+1 is loaded into
@@ -1208,29 +1210,29 @@ k_build_probe(JoinArgs a) {
           if constexpr (PIPE) {
 #pragma unroll
             for (int u = 0; u < JN_U; u++) x[u] = xs[u];
-            if (base + 2 * BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U>(a, base + BATCH, st.s_hi, xs);
+            if (base + 2 * BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, base + BATCH, st.s_hi, xs);
           } else {
-            jn_load_batch<KW, PSW, JN_U>(a, base, st.s_hi, x);
+            jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, base, st.s_hi, x);
           }
-          jn_probe_batch<KW, PRW, PSW, MAT, JN_U>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+          jn_probe_batch<KW, PRW, PSW, MAT, JN_U, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
           base += BATCH;
         }
         const uint32_t rem = st.s_hi > base ? st.s_hi - base : 0;
         if (rem > 2 * JN_CONSUMERS) {
           Tup<KW, PSW> x[4];
-          jn_load_batch<KW, PSW, 4>(a, base, st.s_hi, x);
-          jn_probe_batch<KW, PRW, PSW, MAT, 4>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+          jn_load_batch<KW, PSW, 4, JN_CONSUMERS>(a, base, st.s_hi, x);
+          jn_probe_batch<KW, PRW, PSW, MAT, 4, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
         } else if (rem > JN_CONSUMERS) {
           Tup<KW, PSW> x[2];
-          jn_load_batch<KW, PSW, 2>(a, base, st.s_hi, x);
-          jn_probe_batch<KW, PRW, PSW, MAT, 2>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+          jn_load_batch<KW, PSW, 2, JN_CONSUMERS>(a, base, st.s_hi, x);
+          jn_probe_batch<KW, PRW, PSW, MAT, 2, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
         } else if (rem > 0) {
           Tup<KW, PSW> x[1];
-          jn_load_batch<KW, PSW, 1>(a, base, st.s_hi, x);
-          jn_probe_batch<KW, PRW, PSW, MAT, 1>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+          jn_load_batch<KW, PSW, 1, JN_CONSUMERS>(a, base, st.s_hi, x);
+          jn_probe_batch<KW, PRW, PSW, MAT, 1, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
         }
       }
-      consumer_sync();  // everyone is done with heads/next and ring buffer bi
+      consumer_sync<JN_CONSUMERS>();  // everyone is done with heads/next and ring buffer bi
       if (threadIdx.x == 0) mbar_arrive(&empty[bi]);
     }
   }
