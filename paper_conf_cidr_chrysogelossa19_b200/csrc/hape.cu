@@ -374,16 +374,26 @@ static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, 
 }
 
 // scatter shape per tuple width (measured best of the ScCfg sweep);
-// HAPE_SC=1 selects the destination-table variant (tuning only)
+// (the destination-table variant ScCfg<..., DST=true> is no longer dispatched)
 template <int KW, int PW, bool AOS, bool IDENT, bool CLAIM>
 static hape_status scatter_i(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* offs,
                              void* out) {
   static int v = [] { const char* e = getenv("HAPE_SC"); return e ? atoi(e) : 0; }();
+  // measured (round 1): 8-byte tuples <512,13,2,2> (C2 scatters 1.09/1.03 ->
+  // 0.96/0.93 ms vs the earlier <512,8,3,2>); 16-byte tuples <384,9,2,2>
+  // (C3 7.95/7.04 -> 7.10/6.89 ms vs <256,8,2,3>).  The largest tile two CTAs
+  // per SM can stage wins: longer bucket runs per tile (P585-589: more staged
+  // tuples per partition -> longer runs -> better store coalescing).
+  // HAPE_SC / HAPE_SC16 select the alternatives (tuning only).
   if constexpr (KW + PW <= 8) {
-    if (v == 1) return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2, true>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
-    return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
+    if (v == 1) return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
+    if (v == 2) return scatter_t<KW, PW, AOS, ScCfg<512, 12, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
+    return scatter_t<KW, PW, AOS, ScCfg<512, 13, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
   } else {
-    return scatter_t<KW, PW, AOS, ScCfg<256, 8, 2, 3>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
+    static int w = [] { const char* e = getenv("HAPE_SC16"); return e ? atoi(e) : 0; }();
+    if (w == 1) return scatter_t<KW, PW, AOS, ScCfg<256, 8, 2, 3>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
+    if (w == 2) return scatter_t<KW, PW, AOS, ScCfg<256, 12, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
+    return scatter_t<KW, PW, AOS, ScCfg<384, 9, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
   }
 }
 

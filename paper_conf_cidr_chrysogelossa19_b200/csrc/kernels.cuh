@@ -93,6 +93,22 @@ __device__ __forceinline__ void seg_chunk(const SegMap& m, uint32_t cta, uint32_
   hi = b + (uint32_t)((len * (j + 1)) / m.cps);
 }
 
+// Tile-granular split of a segment (claiming scatters, whose chunking is free):
+// every chunk is whole tiles of T tuples, so only a segment's last tile takes
+// the partial-tile path.
+__device__ __forceinline__ void seg_chunk_tiles(const SegMap& m, uint32_t cta, uint32_t T, uint32_t& seg,
+                                                uint32_t& j, uint32_t& lo, uint32_t& hi) {
+  seg = cta / m.cps;
+  j = cta - seg * m.cps;
+  const uint32_t b = m.bounds ? m.bounds[seg] : 0u;
+  const uint32_t e = m.bounds ? m.bounds[seg + 1] : m.n;
+  const uint32_t len = e - b;
+  const uint64_t nt = (len + (uint64_t)T - 1) / T;
+  const uint64_t t0 = nt * j / m.cps, t1 = nt * (j + 1) / m.cps;
+  lo = b + (uint32_t)(t0 * T < len ? t0 * T : len);
+  hi = b + (uint32_t)(t1 * T < len ? t1 * T : len);
+}
+
 // --------------------------------------------------------------------------
 // small block primitives
 // --------------------------------------------------------------------------
@@ -644,7 +660,8 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
   uint64_t* bar = reinterpret_cast<uint64_t*>(s_wt + 64);
 
   uint32_t seg, j, lo, hi;
-  seg_chunk(m, blockIdx.x, seg, j, lo, hi);
+  if constexpr (CLAIM) seg_chunk_tiles(m, blockIdx.x, (uint32_t)C::T, seg, j, lo, hi);
+  else seg_chunk(m, blockIdx.x, seg, j, lo, hi);
   const bool backward = !CLAIM && (j & 1u) != 0;
   const uint32_t row0 = seg * P;
   const size_t nflat = (size_t)m.nseg * P * m.cps;
