@@ -36,7 +36,10 @@ def launches():
 
 
 def full_metrics(path):
-    out = subprocess.run(["ncu", "-i", path, "--page", "raw", "--csv"], capture_output=True, text=True).stdout
+    if path.endswith(".csv"):  # raw page exported on the GPU box (profile_round.sh)
+        out = open(path).read()
+    else:
+        out = subprocess.run(["ncu", "-i", path, "--page", "raw", "--csv"], capture_output=True, text=True).stdout
     r = list(csv.reader(out.splitlines()))
     res = []
     scale = {"byte": 1, "Kbyte": 1e3, "Mbyte": 1e6, "Gbyte": 1e9, "nsecond": 1, "usecond": 1e3, "msecond": 1e6, "ns": 1, "us": 1e3, "ms": 1e6,
@@ -92,6 +95,8 @@ lines.append("| kernel | us | DRAM rd+wr MB | TB/s | warp inst M | IPC | occ % |
 lines.append("|---|---|---|---|---|---|---|---|---|---|---|---|")
 for name in ("k_hist", "k_hist_joint", "k_scatter", "k_build_probe"):
     path = os.path.join(G, f"full_{TAG}_{CFG}_{name}.ncu-rep")
+    if not os.path.exists(path):
+        path = os.path.join(G, f"full_{TAG}_{CFG}_{name}.raw.csv")
     if not os.path.exists(path):
         continue
     for m in full_metrics(path):

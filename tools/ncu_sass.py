@@ -5,8 +5,12 @@ import csv, subprocess, sys
 
 rep = sys.argv[1]
 minfrac = float(sys.argv[2]) if len(sys.argv) > 2 else 0.002
-out = subprocess.run(["ncu", "-i", rep, "--page", "source", "--csv", "--print-source", "sass"],
-                     capture_output=True, text=True).stdout
+if rep.endswith(".sass.csv.gz"):  # exported on the GPU box by profile_round.sh
+    import gzip
+    out = gzip.open(rep, "rt").read()
+else:
+    out = subprocess.run(["ncu", "-i", rep, "--page", "source", "--csv", "--print-source", "sass"],
+                         capture_output=True, text=True).stdout
 rows = list(csv.reader(out.splitlines()))
 h = rows[1]
 data = [dict(zip(h, r)) for r in rows[2:] if len(r) >= len(h) - 1]

@@ -16,6 +16,12 @@ NH=$((3*2)); NS=$((3*4)); NB=3; HK=k_hist_joint
 if [ "$CFG" = "c1" ]; then NH=6; NS=6; HK=k_hist; fi
 for K in $HK:$NH k_scatter:$NS k_build_probe:$NB; do
   N=${K%%:*}; S=${K##*:}
-  timeout 600 ncu --set full --clock-control none --import-source on -k regex:$N -s $S -c 1 -o gpurun_out/full_${TAG}_${CFG}_${N} $B > /dev/null 2>&1
+  R=gpurun_out/full_${TAG}_${CFG}_${N}
+  timeout 600 ncu --set full --clock-control none --import-source on -k regex:$N -s $S -c 1 -o $R $B > /dev/null 2>&1
+  # exports instead of the report (gpurun returns at most 64 MiB): the raw
+  # metrics page and the per-SASS-line source page
+  ncu -i $R.ncu-rep --page raw --csv > $R.raw.csv 2>/dev/null
+  ncu -i $R.ncu-rep --page source --csv --print-source sass 2>/dev/null | gzip > $R.sass.csv.gz
+  [ -z "$NCU_KEEP_REP" ] && rm -f $R.ncu-rep
 done
 ls -la gpurun_out
