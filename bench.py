@@ -39,6 +39,7 @@ CONFIG_TEXT = {
     "c1": "|R|=|S|=2^20 int32 key/payload, unique PK-FK uniform keys (BASELINE configs[0])",
     "c2": "|R|=|S|=2^27 int32 key/payload, unique uniform keys, 2-pass radix (BASELINE configs[1])",
     "c3": "|R|=2^27, |S|=2^30 int64 key/payload FK join, materialised pairs (BASELINE configs[2])",
+    "c4": "|R|=|S|=2^31 int32, hash-shuffled via NCCL all-to-all and co-partitioned join (BASELINE configs[3])",
 }
 
 
@@ -129,11 +130,13 @@ def run_reference(args):
     rank = int(os.environ.get("RANK", "0"))
     if rank != 0:
         return 0
+    if args.config == "auto":
+        args.config = "c4" if int(os.environ.get("WORLD_SIZE", "1")) > 1 else "c2"
     import numpy as np
     import datagen
     import oracle
     log2n = args.ref_log2n
-    wl = datagen.make(args.config if args.config in ("c1", "c2") else "c2", n_r=1 << log2n, n_s=1 << log2n)
+    wl = datagen.make(args.config if args.config in ("c1", "c2", "c4") else "c2", n_r=1 << log2n, n_s=1 << log2n)
     oracle.build()
     times = []
     for i in range(args.warmup + args.steps):
@@ -148,7 +151,8 @@ def run_reference(args):
     v = n / (ms / 1000)
     line = {"metric": METRIC, "value": v, "unit": UNIT, "impl": "reference", "n_gpus": args.gpus,
             "steps": args.steps, "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True,
-            "scaling": "weak", "vs_baseline": None, "dtype": "int32", "data": "synthetic",
+            "scaling": "strong" if args.config == "c4" else "weak", "vs_baseline": None, "dtype": "int32",
+            "data": "synthetic",
             "config": {"workload": f"{args.config}: CPU oracle on a bounded sample |R|=|S|=2^{log2n} of the same recipe"},
             "cpu_baseline": {"value": v, "unit": UNIT, "cores": oracle.threads_used(), "kind": "oracle",
                              "sample": f"c2 recipe at |R|=|S|=2^{log2n} int32, single-thread sort-merge"},
@@ -163,7 +167,9 @@ def main():
     ap.add_argument("--gpus", type=int, default=1)
     ap.add_argument("--steps", type=int, default=10)
     ap.add_argument("--warmup", type=int, default=3)
-    ap.add_argument("--config", default="c2", choices=["c1", "c2", "c3"])
+    ap.add_argument("--config", default="auto", choices=["auto", "c1", "c2", "c3", "c4"],
+                    help="auto: c2 (BASELINE configs[1]) on one GPU; c4 (2^31 x 2^31 int32, configs[3], "
+                         "sharded over the ranks: strong scaling) under torchrun with N > 1")
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--ref-log2n", type=int, default=22)
     ap.add_argument("--cpu-log2n", type=int, default=24)
@@ -201,8 +207,14 @@ def main():
     args.warmup = max(args.warmup, 3)
 
     cfg = args.config
+    if cfg == "auto":
+        cfg = "c4" if world > 1 else "c2"
     base = datagen.SHAPES[cfg]
-    n_r, n_s = base[0] * world, base[1] * world
+    # c4 is a fixed global job (2^31 per relation) split over the ranks
+    # (strong scaling); the other configs give every rank a full-size shard
+    # of a global relation N times larger (weak scaling)
+    strong = cfg == "c4"
+    n_r, n_s = (base[0], base[1]) if strong else (base[0] * world, base[1] * world)
     wl = datagen.make(cfg, n_r=n_r, n_s=n_s, rank=rank, world=world, backend="torch", device="cuda")
     kdt = torch.int32 if wl.key_bits == 32 else torch.int64
     pdt = torch.int32 if wl.pay_bits == 32 else torch.int64
@@ -448,10 +460,12 @@ def main():
     if rank == 0:
         line = {
             "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
-            "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True, "scaling": "weak",
+            "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True,
+            "scaling": "strong" if strong else "weak",
             "vs_baseline": None, "dtype": "int32" if wl.key_bits == 32 else "int64",
             "data": "synthetic (datagen counter-based recipe, generated on device)",
-            "config": {"workload": f"{cfg}: {CONFIG_TEXT[cfg]}" + (f"; {world} ranks x shard" if world > 1 else "")
+            "config": {"workload": f"{cfg}: {CONFIG_TEXT[cfg]}"
+                       + ((f"; split over {world} ranks" if strong else f"; {world} ranks x shard") if world > 1 else "")
                        + ("; through the 1-rank NCCL exchange path" if (args.exchange and world == 1) else ""),
                        "n_r": n_r, "n_s": n_s, "per_rank_r": nr_loc, "per_rank_s": ns_loc,
                        "passes": res.passes, "bits": list(res.bits), "n_items": res.n_items,
