@@ -884,6 +884,18 @@ k_worklist(const uint32_t* __restrict__ bR, const uint32_t* __restrict__ bS, uin
 // consumer threads per build+probe CTA: a template parameter (JN_CONSUMERS,
 // 256 or 512) of the kernel; one producer warp on top
 constexpr int JN_U = 4;
+#ifndef HAPE_JN_REL_MODE
+#define HAPE_JN_REL_MODE 1
+#endif
+// SR tile release after the consumers' copy to registers: 1 = one consumer
+// barrier, then one arrival (C3 build+probe 10.76 ms; racecheck-clean);
+// 0 = per-warp __syncwarp + lane-0 arrival (10.56 ms; correct by the PTX
+// model's cumulativity, but racecheck cannot see the ordering).  Releasing at
+// the materialising probe's claim barrier instead measured 14.4 ms (the refill
+// starts a whole probe later), and a runtime switch between the forms slowed
+// every form to ~14 ms (a barrier under a runtime branch), so the form is a
+// compile-time choice.
+constexpr int JN_REL = HAPE_JN_REL_MODE;
 constexpr uint32_t JN_MAXCAP = 16384;
 constexpr uint32_t JN_NIL = 0xFFFFu;
 constexpr uint32_t JN_STOP = 0xFFFFFFFFu;
@@ -1111,7 +1123,10 @@ k_build_probe(JoinArgs a) {
 
   if (threadIdx.x == 0) {
     for (uint32_t i = 0; i < NRB; i++) { mbar_init(&full[i], 1); mbar_init(&empty[i], 1); }
-    for (uint32_t i = 0; i < NSB; i++) { mbar_init(&sfull[i], 1); mbar_init(&sempty[i], JN_CONSUMERS / 32); }
+    for (uint32_t i = 0; i < NSB; i++) {
+      mbar_init(&sfull[i], 1);
+      mbar_init(&sempty[i], JN_REL == 0 ? JN_CONSUMERS / 32 : 1);
+    }
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
   }
   __syncthreads();
@@ -1214,8 +1229,14 @@ k_build_probe(JoinArgs a) {
             const uint32_t j = u * JN_CONSUMERS + threadIdx.x;
             if (j < n) x[u] = tile[j];
           }
-          __syncwarp();
-          if (lane == 0) mbar_arrive(&sempty[sb]);
+          // release the tile once every consumer holds its tuples (JN_REL)
+          if constexpr (JN_REL == 0) {
+            __syncwarp();
+            if (lane == 0) mbar_arrive(&sempty[sb]);
+          } else {
+            consumer_sync<JN_CONSUMERS>();
+            if (threadIdx.x == 0) mbar_arrive(&sempty[sb]);
+          }
           jn_probe_batch<KW, PRW, PSW, MAT, XU, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
         }
       } else {

@@ -36,5 +36,14 @@ pin = lambda a: torch.from_numpy(np.ascontiguousarray(a)).pin_memory()
 with RadixJoin(key_dtype=torch.int32) as j:
     res = j.join(pin(wl.R.key), pin(wl.R.payload), pin(wl.S.key), pin(wl.S.payload))
     ok &= res.match_count == want["count"] and res.pair_checksum == want["checksum"]
+# out-of-HBM co-processing: host co-partitioning + per-pair device joins
+wl = datagen.make("c3", n_r=3000, n_s=20000)
+want = oracle.join(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload)
+with RadixJoin(key_dtype=torch.int64) as j:
+    out_r = torch.empty(want["count"], dtype=torch.int64).pin_memory()
+    out_s = torch.empty(want["count"], dtype=torch.int64).pin_memory()
+    res = j.coprocess_join(pin(wl.R.key), pin(wl.R.payload), pin(wl.S.key), pin(wl.S.payload), out_r, out_s,
+                           fanout_bits=2)
+    ok &= res.match_count == want["count"] and res.pair_checksum == want["checksum"]
 _lib.hape_nccl_comm_destroy(comm)
 print("SANITIZE_CASE_OK" if ok else "SANITIZE_CASE_MISMATCH")
