@@ -340,6 +340,33 @@ def test_joint_histogram_row_spill_partitions():
     assert np.array_equal(partition.partition_id(ok, 8, 8), np.repeat(np.arange(1 << 16), np.diff(ob)))
 
 
+def test_joint_histogram_both_halves_of_one_word_wrap():
+    # two hot keys whose joint buckets q (even) and q+1 share one 32-bit
+    # counter word: the low half wraps and carries into the high half, which
+    # wraps too -- the carry fix-up (ovf[q+1] adjustments) must net out exactly
+    n = 1 << 24
+    rng = np.random.default_rng(9)
+    cand = rng.integers(-2**31, 2**31, 200000, dtype=np.int64).astype(np.int32)
+    pid = partition.partition_id(cand, 8, 8)
+    first = {}
+    for k, q in zip(cand.tolist(), pid.tolist()):
+        first.setdefault(int(q), k)
+    q0 = next(q for q in sorted(first) if q % 2 == 0 and q + 1 in first)
+    ka, kb = first[q0], first[q0 + 1]
+    keys = rng.integers(-2**31, 2**31, n, dtype=np.int64).astype(np.int32)
+    u = rng.random(n)
+    keys[u < 0.45] = ka
+    keys[(u >= 0.45) & (u < 0.9)] = kb
+    pays = np.arange(n, dtype=np.int32)
+    j = joiner(torch.int32, radix_passes=2, radix_bits=(8, 8))
+    ok, op, ob, plan = j.debug_partition(cuda(keys), cuda(pays))
+    ok, op, ob = ok.cpu().numpy(), op.cpu().numpy(), ob.cpu().numpy()
+    pid = partition.partition_id(keys, 8, 8)
+    assert np.array_equal(np.diff(ob), np.bincount(pid, minlength=1 << 16))
+    assert np.array_equal(np.sort(op), pays)
+    assert np.array_equal(ok, keys[op.astype(np.int64)])
+
+
 def test_joint_histogram_skewed_join_vs_oracle():
     # the same skew through the join (one S tuple of the hot key: count = its
     # R multiplicity, the R co-partition is joined in chunks)
