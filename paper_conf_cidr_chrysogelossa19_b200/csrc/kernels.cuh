@@ -871,7 +871,7 @@ k_worklist(const uint32_t* __restrict__ bR, const uint32_t* __restrict__ bS, uin
 //     (cp.async.bulk + mbarrier), one "stage" per (R chunk, S slice);
 //   * 8 consumer warps build a chained table over the landed chunk (heads
 //     reset per stage, atomicExch on the heads, u16 next links) and probe the
-//     S slice, streaming S tuples from HBM, 4 independent loads per thread.
+//     S slice, streaming S tuples from HBM, JN_U independent loads per thread.
 // The next stage's R chunk lands while the current one is probed.
 //
 // The slot of a key inside the smem table is a multiplicative hash of the key
@@ -883,7 +883,10 @@ k_worklist(const uint32_t* __restrict__ bR, const uint32_t* __restrict__ bS, uin
 // --------------------------------------------------------------------------
 // consumer threads per build+probe CTA: a template parameter (JN_CONSUMERS,
 // 256 or 512) of the kernel; one producer warp on top
-constexpr int JN_U = 4;
+#ifndef HAPE_JN_U
+#define HAPE_JN_U 2
+#endif
+constexpr int JN_U = HAPE_JN_U;
 #ifndef HAPE_JN_REL_MODE
 #define HAPE_JN_REL_MODE 1
 #endif
