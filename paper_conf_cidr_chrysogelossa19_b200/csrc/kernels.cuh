@@ -398,23 +398,45 @@ k_hist_joint(PartIn in, SegMap m, uint32_t P1, uint32_t P2, uint32_t* __restrict
   // joint bucket = b1 * P2 + b2 = the low B1+B2 bits of h (R3:
   // pass 1 reads bits [B2, B2+B1), pass 2 bits [0, B2))
   const uint32_t qmask = Q - 1;
+  // wrap test: the half is 0xFFFF iff (old | ~(0xFFFF << sh)) is all ones
+  auto wrapped = [](uint32_t q, uint32_t old) -> bool {
+    return (old | ~(0xFFFFu << ((q & 1u) << 4))) == 0xFFFFFFFFu;
+  };
+  auto fixup = [&](uint32_t q, uint32_t old) {  // this increment wrapped its half
+    const uint32_t p = q / P2;
+    atomicAdd(&ovf[q], 65536u);
+    uint32_t dr = 65536u;
+    if (!(q & 1u)) {  // the carry went into the neighbour's half
+      const uint32_t d = (old >> 16) == 0xFFFFu ? 65535u : 0xFFFFFFFFu;
+      atomicAdd(&ovf[q + 1], d);
+      dr += d;
+    }
+    atomicAdd(&rowsum[p], dr);
+  };
+  auto inc = [&](K k, uint32_t& q) -> uint32_t {
+    q = (uint32_t)part_hash<KW, IDENT>(k) & qmask;
+    return atomicAdd(&j16[q >> 1], 1u << ((q & 1u) << 4));
+  };
   auto count = [&](K k) {
-    const uint32_t q = (uint32_t)part_hash<KW, IDENT>(k) & qmask;
-    const uint32_t sh = (q & 1u) << 4;
-    const uint32_t old = atomicAdd(&j16[q >> 1], 1u << sh);
-    // wrap test: the half is 0xFFFF iff (old | ~(0xFFFF << sh)) is all ones;
-    // the rare fix-up runs under a warp-uniform branch
-    const bool wrap = (old | ~(0xFFFFu << sh)) == 0xFFFFFFFFu;
-    if (__any_sync(__activemask(), wrap) && wrap) {  // this increment wrapped its half
-      const uint32_t p = q / P2;
-      atomicAdd(&ovf[q], 65536u);
-      uint32_t dr = 65536u;
-      if (!(q & 1u)) {  // the carry went into the neighbour's half
-        const uint32_t d = (old >> 16) == 0xFFFFu ? 65535u : 0xFFFFFFFFu;
-        atomicAdd(&ovf[q + 1], d);
-        dr += d;
-      }
-      atomicAdd(&rowsum[p], dr);
+    uint32_t q;
+    const uint32_t old = inc(k, q);
+    if (wrapped(q, old)) fixup(q, old);
+  };
+  // the PER keys of one 16-byte vector: all increments issue before any
+  // return value is tested (no atomic round trip per key on the warp's
+  // critical path), one warp vote per vector guards the rare fix-up
+  auto count_vec = [&](const uint4& w) {
+    const E* ee = reinterpret_cast<const E*>(&w);
+    uint32_t q[PER], old[PER];
+#pragma unroll
+    for (int e = 0; e < PER; e++) old[e] = inc(key_of(ee[e]), q[e]);
+    bool any = false;
+#pragma unroll
+    for (int e = 0; e < PER; e++) any |= wrapped(q[e], old[e]);
+    if (__any_sync(__activemask(), any) && any) {
+#pragma unroll
+      for (int e = 0; e < PER; e++)
+        if (wrapped(q[e], old[e])) fixup(q[e], old[e]);
     }
   };
   const uint32_t nchunks = m.nseg * m.cps;
@@ -434,18 +456,9 @@ k_hist_joint(PartIn in, SegMap m, uint32_t P1, uint32_t P2, uint32_t* __restrict
 #pragma unroll
       for (int u = 0; u < HIST_VEC; u++) w[u] = __ldcs(vk + v + u * HJ_THREADS);
 #pragma unroll
-      for (int u = 0; u < HIST_VEC; u++) {
-        const E* ee = reinterpret_cast<const E*>(&w[u]);
-#pragma unroll
-        for (int e = 0; e < PER; e++) count(key_of(ee[e]));
-      }
+      for (int u = 0; u < HIST_VEC; u++) count_vec(w[u]);
     }
-    for (; v < nvec; v += HJ_THREADS) {
-      const uint4 w = __ldcs(vk + v);
-      const E* ee = reinterpret_cast<const E*>(&w);
-#pragma unroll
-      for (int e = 0; e < PER; e++) count(key_of(ee[e]));
-    }
+    for (; v < nvec; v += HJ_THREADS) count_vec(__ldcs(vk + v));
   }
   __syncthreads();
   // row totals of the 16-bit counters: a warp covers 32 consecutive words;
