@@ -7,8 +7,13 @@ A step is one hape_radix_join call over the whole workload: both radix passes
 over R and S (hist -> scan -> scatter), the work list, the smem build+probe
 with the fused count/sum/checksum aggregation and the result read-back.  At
 N=1 the workload is BASELINE.json configs[1] (|R|=|S|=2^27 int32, 2-pass);
-under torchrun (N>1) every rank holds a 2^27-row shard of R and of S of a
-global 2^27*N-row relation (weak scaling), routed by the NCCL exchange.
+under torchrun (N>1) the same c2 workload scales weakly: every rank holds a
+2^27-row shard of R and of S of a global 2^27*N-row relation, routed by the
+NCCL exchange.  `--config c4` runs BASELINE configs[3] (2^31 x 2^31, strong
+scaling: the global job split over the ranks).  At N=1 the line also carries
+`legs`: the other BASELINE configs on the one GPU (C1, C3, C4 = 2^31 x 2^31,
+C2 with the bag-semantics probe, C5 at theta 0.5/0.75/0.9/1.0), each with
+its own stage roofline.
 
 Prints ONE JSON line on rank 0.  `value` is device-resident throughput
 (|R|+|S|)/s; `e2e` repeats the measurement through the same C-ABI call with
@@ -40,6 +45,7 @@ CONFIG_TEXT = {
     "c2": "|R|=|S|=2^27 int32 key/payload, unique uniform keys, 2-pass radix (BASELINE configs[1])",
     "c3": "|R|=2^27, |S|=2^30 int64 key/payload FK join, materialised pairs (BASELINE configs[2])",
     "c4": "|R|=|S|=2^31 int32, hash-shuffled via NCCL all-to-all and co-partitioned join (BASELINE configs[3])",
+    "c5": "|R|=2^28, |S|=2^30 int32 with Zipf-skewed probe keys (BASELINE configs[4])",
 }
 
 
@@ -131,7 +137,7 @@ def run_reference(args):
     if rank != 0:
         return 0
     if args.config == "auto":
-        args.config = "c4" if int(os.environ.get("WORLD_SIZE", "1")) > 1 else "c2"
+        args.config = "c2"
     import numpy as np
     import datagen
     import oracle
@@ -162,14 +168,155 @@ def run_reference(args):
 
 
 # --------------------------------------------------------------------------
+def gen_shard(cfg, n_r, n_s, rank, world, theta=1.0, chunk=1 << 27):
+    """This rank's row shard of config `cfg`, generated on the device in
+    row chunks of <= `chunk` tuples (the torch temporaries of one chunk stay
+    a few GiB even for the 2^31-row C4 relations).  Sub-shards compose
+    exactly: rows [N*i//W, N*(i+1)//W) = the union of the k sub-chunks of
+    rank*k+j over world W*k."""
+    import torch
+    import datagen
+    lo_r, hi_r = (n_r * rank) // world, (n_r * (rank + 1)) // world
+    lo_s, hi_s = (n_s * rank) // world, (n_s * (rank + 1)) // world
+    k = max(1, -(-max(hi_r - lo_r, hi_s - lo_s) // chunk))
+    kw = dict(theta=theta) if cfg == "c5" else {}
+    first = datagen.make(cfg, n_r=n_r, n_s=n_s, rank=rank * k, world=world * k, backend="torch", device="cuda", **kw)
+    if k == 1:
+        return first, [x.contiguous() for x in (first.R.key, first.R.payload, first.S.key, first.S.payload)]
+    cols = [torch.empty(hi_r - lo_r, dtype=first.R.key.dtype, device="cuda"),
+            torch.empty(hi_r - lo_r, dtype=first.R.payload.dtype, device="cuda"),
+            torch.empty(hi_s - lo_s, dtype=first.S.key.dtype, device="cuda"),
+            torch.empty(hi_s - lo_s, dtype=first.S.payload.dtype, device="cuda")]
+    pr = ps = 0
+    for j in range(k):
+        wl = first if j == 0 else datagen.make(cfg, n_r=n_r, n_s=n_s, rank=rank * k + j, world=world * k,
+                                               backend="torch", device="cuda", **kw)
+        a, b = wl.R.n, wl.S.n
+        cols[0][pr:pr + a] = wl.R.key
+        cols[1][pr:pr + a] = wl.R.payload
+        cols[2][ps:ps + b] = wl.S.key
+        cols[3][ps:ps + b] = wl.S.payload
+        pr, ps = pr + a, ps + b
+        del wl
+    assert pr == hi_r - lo_r and ps == hi_s - lo_s
+    return first, cols
+
+
+def alg_bytes(res, kw, prw, psw, materialize, joint):
+    """Algorithmic bytes per stage of one call."""
+    nr, ns = res.r_local, res.s_local
+    tr, ts = kw + prw, kw + psw
+    alg = {"hist1": kw * (nr + ns), "scatter1": 2 * (tr * nr + ts * ns),
+           "hist2": kw * (nr + ns), "scatter2": 2 * (tr * nr + ts * ns),
+           "build_probe": tr * nr + ts * ns + ((prw + psw) * res.n_written if materialize else 0)}
+    if joint:
+        alg.pop("hist2")
+    if res.passes < 2:
+        alg.pop("hist2", None)
+        alg.pop("scatter2")
+    return alg
+
+
+KERNEL_NAME = {"hist1": "k_hist pass 1 (R+S)", "scatter1": "k_scatter pass 1 (R+S)",
+               "hist2": "k_hist pass 2 (R+S)", "scatter2": "k_scatter pass 2 (R+S)",
+               "build_probe": "k_build_probe", "devpart": "device partition (hist+scan+scatter)"}
+
+
+def is_joint(res):
+    return (res.passes == 2 and 6 <= res.bits[0] + res.bits[1] <= 16
+            and os.environ.get("HAPE_JOINT", "1") != "0")
+
+
+def roofline_of(res, stage_avg, ms, kw, prw, psw, materialize, peak, extra=None):
+    joint = is_joint(res)
+    alg = alg_bytes(res, kw, prw, psw, materialize, joint)
+    alg.update(extra or {})
+    per_stage = {}
+    for k in alg:
+        if stage_avg.get(k, 0) > 0:
+            gbs = alg[k] / (stage_avg[k] / 1000.0) / 1e9
+            per_stage[k] = {"ms": round(stage_avg[k], 4), "alg_bytes": alg[k], "GB/s": round(gbs, 1),
+                            "frac": round(gbs / peak, 3)}
+    dom = max(per_stage, key=lambda k: per_stage[k]["ms"])
+    names = dict(KERNEL_NAME)
+    if joint:
+        names["hist1"] = "k_hist_joint (pass-1 and pass-2 buckets, R+S)"
+        names["scatter1"] = "k_scatter pass 1, claiming (R+S)"
+        names["scatter2"] = "k_scatter pass 2, claiming (R+S)"
+    alg_total = sum(alg.values())
+    return {"bound": "hbm", "achieved": per_stage[dom]["GB/s"], "peak": peak, "unit": "GB/s",
+            "frac": round(per_stage[dom]["GB/s"] / peak, 4), "kernel": names[dom], "dominant_stage": dom,
+            "step": {"alg_bytes": alg_total, "GB/s": round(alg_total / (ms / 1000) / 1e9, 1),
+                     "frac": round(alg_total / (ms / 1000) / 1e9 / peak, 4)},
+            "stages": per_stage}
+
+
+def time_calls(fn, steps, stream):
+    """CUDA events on the library's stream around `steps` calls; returns
+    (ms per call, summed stage_ms, launches, last result)."""
+    import torch
+    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+    stage_sum, launches, res = {}, 0, None
+    e0.record(stream)
+    for _ in range(steps):
+        res = fn()
+        launches += res.kernel_launches
+        for k, v in res.stage_ms.items():
+            stage_sum[k] = stage_sum.get(k, 0.0) + v
+    e1.record(stream)
+    torch.cuda.synchronize()
+    return e0.elapsed_time(e1) / steps, {k: v / steps for k, v in stage_sum.items()}, launches, res
+
+
+def run_leg(name, cfg, args, peak, n_r=None, n_s=None, theta=1.0, r_unique=True, materialize=None, steps=None):
+    """One extra single-GPU workload (a bench 'leg'): generate, warm up, time."""
+    import torch
+    import datagen
+    from paper_conf_cidr_chrysogelossa19_b200 import RadixJoin
+    base = datagen.SHAPES[cfg]
+    n_r = n_r or base[0]
+    n_s = n_s or base[1]
+    t0 = time.perf_counter()
+    wl, (rk, rp, sk, sp) = gen_shard(cfg, n_r, n_s, 0, 1, theta=theta)
+    gen_s = time.perf_counter() - t0
+    mat = (cfg == "c3") if materialize is None else materialize
+    out_r = out_s = None
+    if mat:
+        out_r = torch.empty(n_s, dtype=rp.dtype, device="cuda")
+        out_s = torch.empty(n_s, dtype=sp.dtype, device="cuda")
+    j = RadixJoin(key_dtype=rk.dtype, r_payload_dtype=rp.dtype, s_payload_dtype=sp.dtype,
+                  max_r=n_r, max_s=n_s, r_unique=r_unique, stream=torch.cuda.current_stream())
+    for _ in range(args.warmup):
+        res = j.join(rk, rp, sk, sp, out_r, out_s)
+    torch.cuda.synchronize()
+    k = steps or args.leg_steps
+    ms, st, launches, res = time_calls(lambda: j.join(rk, rp, sk, sp, out_r, out_s), k, j.stream)
+    kw, prw, psw = rk.element_size(), rp.element_size(), sp.element_size()
+    roof = roofline_of(res, st, ms, kw, prw, psw, mat, peak)
+    leg = {"workload": f"{cfg}: {CONFIG_TEXT.get(cfg, cfg)}" + (f"; theta={theta}" if cfg == "c5" else "")
+           + ("" if r_unique else "; bag-semantics probe (R not declared unique)"),
+           "n_r": n_r, "n_s": n_s, "steps": k, "ms_per_step": round(ms, 4), "value": (n_r + n_s) / (ms / 1000.0),
+           "unit": UNIT, "passes": res.passes, "bits": list(res.bits), "n_items": res.n_items,
+           "match_count": res.match_count, "r_unique_declared": r_unique, "materialize": mat,
+           "gpu_launches": launches, "gen_s": round(gen_s, 2), "roofline": roof}
+    if cfg in ("c1", "c2", "c4") and n_s == n_r:
+        leg["count_ok"] = res.match_count == n_s   # PK-FK same key set: |J| = |S| (P793-794)
+    if cfg in ("c3", "c5"):
+        leg["count_ok"] = res.match_count == n_s   # FK: every S key is in R
+    j.close()
+    del rk, rp, sk, sp, out_r, out_s, wl
+    torch.cuda.empty_cache()
+    return leg
+
+
 def main():
     ap = argparse.ArgumentParser()
     ap.add_argument("--gpus", type=int, default=1)
     ap.add_argument("--steps", type=int, default=10)
     ap.add_argument("--warmup", type=int, default=3)
-    ap.add_argument("--config", default="auto", choices=["auto", "c1", "c2", "c3", "c4"],
-                    help="auto: c2 (BASELINE configs[1]) on one GPU; c4 (2^31 x 2^31 int32, configs[3], "
-                         "sharded over the ranks: strong scaling) under torchrun with N > 1")
+    ap.add_argument("--config", default="auto", choices=["auto", "c1", "c2", "c3", "c4", "c5"],
+                    help="auto: c2 (BASELINE configs[1]) at every N: one GPU runs |R|=|S|=2^27, N ranks "
+                         "each hold a 2^27-row shard of R and of S of a global 2^27*N relation (weak scaling)")
     ap.add_argument("--impl", default="ours", choices=["ours", "reference"])
     ap.add_argument("--ref-log2n", type=int, default=22)
     ap.add_argument("--cpu-log2n", type=int, default=24)
@@ -181,6 +328,11 @@ def main():
     ap.add_argument("--no-mat", action="store_true", help="c3 without materialised pairs (diagnostics)")
     ap.add_argument("--bag", action="store_true",
                     help="do not declare R's keys unique (HAPE_FLAG_R_UNIQUE): full bag-semantics probe")
+    ap.add_argument("--theta", type=float, default=1.0, help="c5 Zipf skew")
+    ap.add_argument("--legs", default="default",
+                    help="extra single-GPU workloads at N=1, comma list of c1,c3,c4,c2bag,c5 (or c5:THETA); "
+                         "'default' = c1,c3,c4,c2bag,c5:0.5,c5:0.75,c5:0.9,c5:1.0; 'none'")
+    ap.add_argument("--leg-steps", type=int, default=5)
     ap.add_argument("--no-ablation", action="store_true",
                     help="skip the non-partitioned GPU join comparison (PAPER.md Fig. 6)")
     ap.add_argument("--no-coprocess", action="store_true",
@@ -202,23 +354,26 @@ def main():
     rank = int(os.environ.get("RANK", "0"))
     local = int(os.environ.get("LOCAL_RANK", "0"))
     torch.cuda.set_device(local)
+    # one non-default stream for everything: the generator's kernels, the
+    # library's kernels and the timing events are ordered on it
+    stream = torch.cuda.Stream()
+    torch.cuda.set_stream(stream)
     if world > 1:
         dist.init_process_group("nccl", device_id=torch.device("cuda", local))
     args.warmup = max(args.warmup, 3)
+    peak, peak_src = load_peaks()
 
     cfg = args.config
     if cfg == "auto":
-        cfg = "c4" if world > 1 else "c2"
+        cfg = "c2"
     base = datagen.SHAPES[cfg]
     # c4 is a fixed global job (2^31 per relation) split over the ranks
     # (strong scaling); the other configs give every rank a full-size shard
     # of a global relation N times larger (weak scaling)
     strong = cfg == "c4"
     n_r, n_s = (base[0], base[1]) if strong else (base[0] * world, base[1] * world)
-    wl = datagen.make(cfg, n_r=n_r, n_s=n_s, rank=rank, world=world, backend="torch", device="cuda")
-    kdt = torch.int32 if wl.key_bits == 32 else torch.int64
-    pdt = torch.int32 if wl.pay_bits == 32 else torch.int64
-    rk, rp, sk, sp = (x.contiguous() for x in (wl.R.key, wl.R.payload, wl.S.key, wl.S.payload))
+    wl, (rk, rp, sk, sp) = gen_shard(cfg, n_r, n_s, rank, world, theta=args.theta)
+    kdt, pdt = rk.dtype, rp.dtype
     nr_loc, ns_loc = rk.shape[0], sk.shape[0]
     materialize = cfg == "c3" and not args.no_mat
 
@@ -229,12 +384,11 @@ def main():
             dist.broadcast_object_list(uid, src=0)
         st, comm = _lib.hape_nccl_comm_init(uid[0], world, rank, local)
         assert st == 0, f"nccl comm init failed: {st}"
-    stream = torch.cuda.current_stream()
     j = RadixJoin(key_dtype=kdt, r_payload_dtype=pdt, s_payload_dtype=pdt, device=local,
                   max_r=nr_loc, max_s=ns_loc, world_size=world, rank=rank,
                   radix_passes=args.passes, radix_bits=tuple(int(x) for x in args.bits.split(",")),
-                  r_unique=not args.bag,
-                  nccl_comm=comm, stream=stream)
+                  r_unique=not args.bag, nccl_comm=comm, stream=stream)
+    assert j.stream.cuda_stream == stream.cuda_stream
     out_r = out_s = None
     if materialize:
         cap = int(ns_loc * 1.1) if world > 1 else ns_loc
@@ -259,86 +413,43 @@ def main():
     verify = None
     if args.verify and world == 1:
         from oracle import provenance
-        import numpy as np
-        want = provenance.expected_pkfk(wl.R.payload[wl.idx].cpu().numpy(), wl.S.payload.cpu().numpy())
-        verify = (res.match_count, res.sum_r_payload, res.sum_s_payload, res.pair_checksum) == \
-            (want["count"], want["sum_r"], want["sum_s"], want["checksum"])
+        want = provenance.expected_pkfk(wl.R.payload[wl.idx].cpu().numpy(), wl.S.payload.cpu().numpy()) \
+            if wl.idx is not None and n_r == wl.R.n else None
+        if want is not None:
+            verify = (res.match_count, res.sum_r_payload, res.sum_s_payload, res.pair_checksum) == \
+                (want["count"], want["sum_r"], want["sum_s"], want["checksum"])
     clocks = ClockSampler(local)
     barrier()
     clocks.start()
     time.sleep(0.3)
     barrier()
-    e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
-    stage_sum = {}
-    launches = 0
-    e0.record(stream)
-    for _ in range(args.steps):
-        res = j.join(rk, rp, sk, sp, out_r, out_s)
-        launches += res.kernel_launches
-        for k, v in res.stage_ms.items():
-            stage_sum[k] = stage_sum.get(k, 0.0) + v
-    e1.record(stream)
+    ms_loc, stage_avg, launches, res = time_calls(lambda: j.join(rk, rp, sk, sp, out_r, out_s), args.steps, stream)
     barrier()
     clk = clocks.stop()
-    ms = max_over_ranks(e0.elapsed_time(e1) / args.steps)
+    ms = max_over_ranks(ms_loc)
     total_tuples = n_r + n_s
     value = total_tuples / (ms / 1000.0)
-    stage_avg = {k: v / args.steps for k, v in stage_sum.items()}
 
     # ---- roofline of the dominant kernel stage (algorithmic bytes)
-    kw = wl.key_bits // 8
-    pw = wl.pay_bits // 8
+    kw, pw = rk.element_size(), rp.element_size()
     t = kw + pw
-    nr_j, ns_j = res.r_local, res.s_local
-    alg = {
-        "hist1": kw * (nr_j + ns_j), "scatter1": 2 * t * (nr_j + ns_j),
-        "hist2": kw * (nr_j + ns_j), "scatter2": 2 * t * (nr_j + ns_j),
-        "build_probe": t * (nr_j + ns_j) + (2 * pw * res.n_written if materialize else 0),
-        "devpart": (kw + 2 * t) * (nr_loc + ns_loc),
-    }
-    # two-pass plans with bits[0]+bits[1] <= 16 count both passes' buckets in
-    # the one read of the keys (k_hist_joint, stage hist1); k_joint_reduce
-    # (stage scan1, a few MB of per-SM partials) gives both passes' bounds and
-    # both scatters claim their runs: there is no pass-2 histogram read
-    joint = (res.passes == 2 and 6 <= res.bits[0] + res.bits[1] <= 16
-             and os.environ.get("HAPE_JOINT", "1") != "0")
-    kernel_name = {"hist1": "k_hist pass 1 (R+S)", "scatter1": "k_scatter pass 1 (R+S)",
-                   "hist2": "k_hist pass 2 (R+S)", "scatter2": "k_scatter pass 2 (R+S)",
-                   "build_probe": "k_build_probe", "devpart": "device partition (hist+scan+scatter)"}
-    if joint:
-        alg.pop("hist2")
-        kernel_name["hist1"] = "k_hist_joint (pass-1 and pass-2 buckets, R+S)"
-        kernel_name["scatter1"] = "k_scatter pass 1, claiming (R+S)"
-        kernel_name["scatter2"] = "k_scatter pass 2, claiming (R+S)"
-    if res.passes < 2:
-        alg.pop("hist2", None); alg.pop("scatter2")
-    dom = max((k for k in alg if stage_avg.get(k, 0) > 0), key=lambda k: stage_avg[k])
-    peak, peak_src = load_peaks()
-    per_stage = {}
-    for k in alg:
-        if stage_avg.get(k, 0) > 0:
-            gbs = alg[k] / (stage_avg[k] / 1000.0) / 1e9
-            per_stage[k] = {"ms": round(stage_avg[k], 4), "alg_bytes": alg[k], "GB/s": round(gbs, 1),
-                            "frac": round(gbs / peak, 3)}
+    extra = {}
+    if world > 1 or args.exchange:
+        extra["devpart"] = (kw + 2 * t) * (nr_loc + ns_loc)
+    roofline = roofline_of(res, stage_avg, ms, kw, pw, pw, materialize, peak, extra)
+    roofline["peak_source"] = peak_src
     traffic = None
     try:
         tj = json.load(open(os.path.join(ROOT, "profiles", "ncu_traffic.json")))
-        traffic = tj.get(cfg, {}).get(dom)
+        traffic = tj.get(cfg, {}).get(roofline["dominant_stage"])
     except Exception:
         pass
-    achieved = per_stage[dom]["GB/s"]
-    alg_total = sum(alg[k] for k in alg if k != "devpart") + (alg["devpart"] if (world > 1 or args.exchange) else 0)
+    roofline["traffic"] = traffic
     if stage_avg.get("exchange", 0) > 0:
         xb = t * (nr_loc + ns_loc)  # every local tuple leaves through the exchange (incl. the self segment)
-        per_stage["exchange"] = {"ms": round(stage_avg["exchange"], 4), "bytes_sent": xb,
-                                 "GB/s": round(xb / (stage_avg["exchange"] / 1000.0) / 1e9, 1),
-                                 "bound": "nvlink (NCCL all-to-allv)"}
-    roofline = {"bound": "hbm", "achieved": achieved, "peak": peak, "unit": "GB/s",
-                "frac": round(achieved / peak, 4), "traffic": traffic, "kernel": kernel_name[dom],
-                "peak_source": peak_src,
-                "step": {"alg_bytes": alg_total, "GB/s": round(alg_total / (ms / 1000) / 1e9, 1),
-                         "frac": round(alg_total / (ms / 1000) / 1e9 / peak, 4)},
-                "stages": per_stage}
+        roofline["stages"]["exchange"] = {"ms": round(stage_avg["exchange"], 4), "bytes_sent": xb,
+                                          "GB/s": round(xb / (stage_avg["exchange"] / 1000.0) / 1e9, 1),
+                                          "bound": "nvlink (NCCL all-to-allv)"}
 
     # ---- end to end through the same C ABI call with pinned host buffers
     e2e = None
@@ -351,7 +462,7 @@ def main():
         for _ in range(2):
             j.join(*hk, *(ho or (None, None)))
         barrier()
-        t0 = time.perf_counter()
+        e0, e1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
         e0.record(stream)
         n_e2e = max(1, min(args.steps, 5))
         d2h = 0
@@ -436,19 +547,39 @@ def main():
         for _ in range(2):
             rn = j.join_nonpartitioned(rk, rp, sk, sp, out_r, out_s)
         barrier()
-        e0.record(stream)
-        n_np = max(1, min(args.steps, 5))
-        for _ in range(n_np):
-            rn = j.join_nonpartitioned(rk, rp, sk, sp, out_r, out_s)
-        e1.record(stream)
-        barrier()
-        np_ms = e0.elapsed_time(e1) / n_np
+        np_ms, _, _, rn = time_calls(lambda: j.join_nonpartitioned(rk, rp, sk, sp, out_r, out_s),
+                                     max(1, min(args.steps, 5)), stream)
         nonpart = {"method": "non-partitioned GPU hash join (hape_nonpartitioned_join, PAPER.md Fig. 6 baseline)",
                    "ms_per_step": round(np_ms, 4), "value": total_tuples / (np_ms / 1000.0), "unit": UNIT,
                    "radix_speedup": round(np_ms / ms, 3),
                    "stages_ms": {"build (clear + insert)": round(rn.stage_ms["np_build"], 4),
                                  "probe": round(rn.stage_ms["np_probe"], 4)},
                    "same_result_as_radix": rn.as_tuple() == res.as_tuple()}
+
+    j.close()
+    del rk, rp, sk, sp, out_r, out_s
+    torch.cuda.empty_cache()
+
+    # ---- the other BASELINE configs on this one GPU (extra keys of the line)
+    legs = {}
+    if world == 1 and args.legs != "none":
+        spec = args.legs if args.legs != "default" else "c1,c3,c4,c2bag,c5:0.5,c5:0.75,c5:0.9,c5:1.0"
+        for item in [x for x in spec.split(",") if x]:
+            try:
+                if item == "c2bag":
+                    legs[item] = run_leg(item, "c2", args, peak, r_unique=False)
+                elif item.startswith("c5"):
+                    th = float(item.split(":")[1]) if ":" in item else 1.0
+                    legs[f"c5_theta{th}"] = run_leg(item, "c5", args, peak, theta=th)
+                else:
+                    legs[item] = run_leg(item, item, args, peak, steps=args.leg_steps if item != "c1" else 50)
+            except Exception as ex:  # never lose the main line to a leg
+                legs[item] = {"error": repr(ex)[:400]}
+                torch.cuda.empty_cache()
+        if "c5_theta1.0" in legs and "c5_theta0.5" in legs and "ms_per_step" in legs["c5_theta1.0"] \
+                and "ms_per_step" in legs.get("c5_theta0.5", {}):
+            legs["c5_skew_ratio_theta1_vs_0.5"] = round(legs["c5_theta1.0"]["ms_per_step"]
+                                                        / legs["c5_theta0.5"]["ms_per_step"], 3)
 
     cpu = None
     if rank == 0 and world == 1 and not args.no_cpu_baseline:
@@ -462,7 +593,7 @@ def main():
             "metric": METRIC, "value": value, "unit": UNIT, "n_gpus": world, "steps": args.steps,
             "warmup": args.warmup, "ms_per_step": ms, "higher_is_better": True,
             "scaling": "strong" if strong else "weak",
-            "vs_baseline": None, "dtype": "int32" if wl.key_bits == 32 else "int64",
+            "vs_baseline": None, "dtype": "int32" if kdt == torch.int32 else "int64",
             "data": "synthetic (datagen counter-based recipe, generated on device)",
             "config": {"workload": f"{cfg}: {CONFIG_TEXT[cfg]}"
                        + ((f"; split over {world} ranks" if strong else f"; {world} ranks x shard") if world > 1 else "")
@@ -483,10 +614,11 @@ def main():
             line["nonpartitioned_gpu"] = nonpart
         if coproc is not None:
             line["coprocess"] = coproc
+        if legs:
+            line["legs"] = legs
         if verify is not None:
             line["verified_vs_provenance"] = verify
         print(json.dumps(line), flush=True)
-    j.close()
     if comm is not None:
         _lib.hape_nccl_comm_destroy(comm)
     if world > 1:

@@ -22,11 +22,12 @@ from ._lib import (HAPE_INT32, HAPE_INT64, HAPE_MEM_DEVICE, HAPE_MEM_HOST, HAPE_
                    hape_join_result, hape_last_error, hape_output, hape_radix_join,
                    hape_nonpartitioned_join, hape_coprocess_join, hape_coprocess_config,
                    hape_host_partition,
-                   hape_relation, hape_status_string, hape_debug_partition, hape_version)
+                   hape_relation, hape_status_string, hape_debug_partition, hape_version,
+                   hape_join_stream, hape_debug_route, hape_debug_loopback_join)
 
 __all__ = ["RadixJoin", "JoinResult", "HapeError", "hape_version", "hape_join_create",
            "hape_radix_join", "hape_nonpartitioned_join", "hape_coprocess_join", "hape_join_destroy",
-           "host_partition", "STAGES"]
+           "hape_join_stream", "hape_debug_route", "hape_debug_loopback_join", "host_partition", "STAGES"]
 
 
 class HapeError(RuntimeError):
@@ -70,16 +71,35 @@ def _dt(torch_dtype) -> int:
     raise TypeError(f"unsupported dtype {torch_dtype} (int32 / int64 only)")
 
 
-def _rel(key, pay) -> hape_relation:
+def _rel(key, pay, key_type=None, pay_type=None, device=None) -> hape_relation:
     if key.dim() != 1 or pay.dim() != 1 or key.shape[0] != pay.shape[0]:
         raise ValueError("key/payload must be 1-D columns of equal length")
     if not key.is_contiguous() or not pay.is_contiguous():
         raise ValueError("columns must be contiguous")
-    if key.device.type != pay.device.type:
-        raise ValueError("key and payload must live on the same device type")
+    if key.device != pay.device:
+        raise ValueError("key and payload must live on the same device")
+    if key_type is not None and _dt(key.dtype) != key_type:
+        raise ValueError(f"key dtype {key.dtype} does not match the handle's key type")
+    if pay_type is not None and _dt(pay.dtype) != pay_type:
+        raise ValueError(f"payload dtype {pay.dtype} does not match the handle's payload type")
+    if key.is_cuda and device is not None and key.device.index != device:
+        raise ValueError(f"columns live on {key.device}, the handle on cuda:{device}")
     mem = HAPE_MEM_DEVICE if key.is_cuda else HAPE_MEM_HOST
     return hape_relation(key.data_ptr() if key.numel() else None,
                          pay.data_ptr() if pay.numel() else None, key.shape[0], mem)
+
+
+def _result(st, res) -> "JoinResult":
+    return JoinResult(
+        status=st, match_count=res.match_count, sum_r_payload=res.sum_r_payload,
+        sum_s_payload=res.sum_s_payload, pair_checksum=res.pair_checksum,
+        local_match_count=res.local_match_count, local_sum_r=res.local_sum_r,
+        local_sum_s=res.local_sum_s, local_pair_checksum=res.local_pair_checksum,
+        n_written=res.n_written, n_required=res.n_required, r_local=res.r_local,
+        s_local=res.s_local, passes=res.passes, bits=(res.bits[0], res.bits[1]),
+        n_partitions=res.n_partitions, n_items=res.n_items,
+        kernel_launches=res.kernel_launches,
+        stage_ms={name: float(res.stage_ms[i]) for i, name in enumerate(STAGES)})
 
 
 class RadixJoin:
@@ -108,12 +128,16 @@ class RadixJoin:
         if stream is None:
             stream = torch.cuda.current_stream(device)
         cfg.stream = stream.cuda_stream if hasattr(stream, "cuda_stream") else int(stream)
-        self._stream_handle = cfg.stream
         self.cfg = cfg
         st, h = hape_join_create(cfg)
         if st != HAPE_OK:
             raise HapeError(st, "hape_join_create failed")
         self._h = h
+        # the stream the library really enqueues on (a NULL stream -- torch's
+        # legacy default stream -- makes the handle create its own)
+        st, self._stream_handle = hape_join_stream(h)
+        if st != HAPE_OK:
+            raise HapeError(st, "hape_join_stream failed")
 
     def close(self):
         if getattr(self, "_h", None) is not None and self._h.value:
@@ -143,12 +167,22 @@ class RadixJoin:
         return p
 
     def _order_inputs(self):
-        """Inputs produced on another torch stream must be complete before the
-        library's stream reads them (the ABI leaves ordering to the caller)."""
+        """Order the library's stream after torch's current stream: inputs
+        produced there must be complete before the join's kernels read them
+        (the ABI leaves ordering to the caller, include/hape.h)."""
         import torch
-        cur = torch.cuda.current_stream(self.cfg.device)
+        dev = self.cfg.device
+        cur = torch.cuda.current_stream(dev)
         if cur.cuda_stream != self._stream_handle:
-            cur.synchronize()
+            ev = torch.cuda.Event()
+            ev.record(cur)
+            torch.cuda.ExternalStream(self._stream_handle, device=dev).wait_event(ev)
+
+    @property
+    def stream(self):
+        """The library's stream as a torch stream object."""
+        import torch
+        return torch.cuda.ExternalStream(self._stream_handle, device=self.cfg.device)
 
     def join(self, rk, rp, sk, sp, out_r=None, out_s=None, raise_on_capacity: bool = True) -> JoinResult:
         """hape_radix_join: the partitioned radix hash join (the product path)."""
@@ -171,37 +205,81 @@ class RadixJoin:
         fn = lambda h, R, S, out, res: hape_coprocess_join(h, R, S, cp, out, res)  # noqa: E731
         return self._call(fn, rk, rp, sk, sp, out_r, out_s, raise_on_capacity)
 
+    def _rels(self, rk, rp, sk, sp):
+        c = self.cfg
+        R = _rel(rk, rp, c.key_type, c.r_payload_type, c.device)
+        S = _rel(sk, sp, c.key_type, c.s_payload_type, c.device)
+        return R, S
+
+    def _out(self, out_r, out_s):
+        if out_r is None and out_s is None:
+            return None
+        c = self.cfg
+        if out_r is None or out_s is None or out_r.dim() != 1 or out_s.dim() != 1 \
+                or out_r.shape[0] != out_s.shape[0]:
+            raise ValueError("out_r / out_s must be given together as 1-D tensors of equal length")
+        if not out_r.is_contiguous() or not out_s.is_contiguous():
+            raise ValueError("out_r / out_s must be contiguous")
+        if out_r.device != out_s.device:
+            raise ValueError("out_r / out_s must live on the same device")
+        if _dt(out_r.dtype) != c.r_payload_type or _dt(out_s.dtype) != c.s_payload_type:
+            raise ValueError("out_r / out_s dtypes must match the R / S payload types")
+        if out_r.is_cuda and out_r.device.index != c.device:
+            raise ValueError(f"outputs live on {out_r.device}, the handle on cuda:{c.device}")
+        return hape_output(out_r.data_ptr(), out_s.data_ptr(), out_r.shape[0],
+                           HAPE_MEM_DEVICE if out_r.is_cuda else HAPE_MEM_HOST)
+
     def _call(self, fn, rk, rp, sk, sp, out_r, out_s, raise_on_capacity) -> JoinResult:
+        R, S = self._rels(rk, rp, sk, sp)
+        out = self._out(out_r, out_s)
         self._order_inputs()
-        R = _rel(rk, rp)
-        S = _rel(sk, sp)
-        out = None
-        if out_r is not None:
-            if out_s is None or out_r.shape[0] != out_s.shape[0]:
-                raise ValueError("out_r / out_s must be given together with equal length")
-            out = hape_output(out_r.data_ptr(), out_s.data_ptr(), out_r.shape[0],
-                              HAPE_MEM_DEVICE if out_r.is_cuda else HAPE_MEM_HOST)
         res = hape_join_result()
         st = fn(self._h, R, S, out, res)
         if st != HAPE_OK and not (st == HAPE_ERR_OUTPUT_CAPACITY and not raise_on_capacity):
             raise HapeError(st, hape_last_error(self._h))
-        return JoinResult(
-            status=st, match_count=res.match_count, sum_r_payload=res.sum_r_payload,
-            sum_s_payload=res.sum_s_payload, pair_checksum=res.pair_checksum,
-            local_match_count=res.local_match_count, local_sum_r=res.local_sum_r,
-            local_sum_s=res.local_sum_s, local_pair_checksum=res.local_pair_checksum,
-            n_written=res.n_written, n_required=res.n_required, r_local=res.r_local,
-            s_local=res.s_local, passes=res.passes, bits=(res.bits[0], res.bits[1]),
-            n_partitions=res.n_partitions, n_items=res.n_items,
-            kernel_launches=res.kernel_launches,
-            stage_ms={name: float(res.stage_ms[i]) for i, name in enumerate(STAGES)})
+        return _result(st, res)
+
+    def loopback_join(self, r_shards, s_shards, out_r=None, out_s=None, raise_on_capacity: bool = True):
+        """hape_debug_loopback_join: len(r_shards) simulated ranks on this GPU
+        (every device step of the G>1 path; device copies stand in for NCCL).
+        r_shards / s_shards: lists of (key, payload) CUDA tensor pairs.
+        Returns (total JoinResult, [per-destination JoinResult])."""
+        G = len(r_shards)
+        if len(s_shards) != G:
+            raise ValueError("one R and one S shard per simulated rank")
+        rels = [self._rels(rk, rp, sk, sp) for (rk, rp), (sk, sp) in zip(r_shards, s_shards)]
+        out = self._out(out_r, out_s)
+        self._order_inputs()
+        per = (hape_join_result * G)()
+        tot = hape_join_result()
+        st = hape_debug_loopback_join(self._h, G, [r for r, _ in rels], [s for _, s in rels], out, per, tot)
+        if st != HAPE_OK and not (st == HAPE_ERR_OUTPUT_CAPACITY and not raise_on_capacity):
+            raise HapeError(st, hape_last_error(self._h))
+        return _result(st, tot), [_result(st, per[d]) for d in range(G)]
+
+    def debug_route(self, key, pay, fanout: int, is_s: bool = False):
+        """hape_debug_route: the destination partition with fan-out `fanout`;
+        returns (keys, payloads, bounds[int64 of fanout+1])."""
+        import torch
+        c = self.cfg
+        rel = _rel(key, pay, c.key_type, c.s_payload_type if is_s else c.r_payload_type, c.device)
+        self._order_inputs()
+        dev = torch.device("cuda", c.device)
+        ok = torch.empty_like(key, device=dev)
+        op = torch.empty_like(pay, device=dev)
+        ob = torch.empty(fanout + 1, dtype=torch.int32, device=dev)
+        st = hape_debug_route(self._h, rel, int(is_s), int(fanout), ok.data_ptr(), op.data_ptr(), ob.data_ptr())
+        if st != HAPE_OK:
+            raise HapeError(st, hape_last_error(self._h))
+        return ok, op, ob.to(torch.int64) & 0xFFFFFFFF
 
     def debug_partition(self, key, pay, is_s: bool = False, plan=None):
         """Run the planned radix passes on one relation; returns
         (partitioned keys, partitioned payloads, bounds[int64], plan)."""
         import torch
+        c = self.cfg
+        rel = _rel(key, pay, c.key_type, c.s_payload_type if is_s else c.r_payload_type, c.device)
         self._order_inputs()
-        rel = _rel(key, pay)
         dev = torch.device("cuda", self.cfg.device)
         ok = torch.empty_like(key, device=dev)
         op = torch.empty_like(pay, device=dev)

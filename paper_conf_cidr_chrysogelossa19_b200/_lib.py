@@ -36,7 +36,7 @@ EXPORTED = ["hape_version", "hape_status_string", "hape_join_create", "hape_radi
             "hape_join_destroy", "hape_last_error", "hape_join_plan", "hape_debug_partition",
             "hape_nccl_unique_id", "hape_nccl_comm_init", "hape_nccl_comm_destroy",
             "hape_exchange_plan", "hape_nonpartitioned_join", "hape_coprocess_join",
-            "hape_host_partition"]
+            "hape_host_partition", "hape_join_stream", "hape_debug_route", "hape_debug_loopback_join"]
 
 
 class hape_join_config(ctypes.Structure):
@@ -126,6 +126,13 @@ def _load() -> ctypes.CDLL:
     lib.hape_exchange_plan.restype = ctypes.c_int
     lib.hape_exchange_plan.argtypes = [ctypes.c_int, ctypes.c_int, P(ctypes.c_uint64),
                                        P(ctypes.c_uint64), P(ctypes.c_uint64), P(ctypes.c_uint64)]
+    lib.hape_join_stream.restype = ctypes.c_int
+    lib.hape_join_stream.argtypes = [vp, P(vp)]
+    lib.hape_debug_route.restype = ctypes.c_int
+    lib.hape_debug_route.argtypes = [vp, P(hape_relation), ctypes.c_int, ctypes.c_int, vp, vp, vp]
+    lib.hape_debug_loopback_join.restype = ctypes.c_int
+    lib.hape_debug_loopback_join.argtypes = [vp, ctypes.c_int, P(hape_relation), P(hape_relation),
+                                             P(hape_output), P(hape_join_result), P(hape_join_result)]
     return lib
 
 
@@ -220,3 +227,21 @@ def hape_exchange_plan(world: int, rank: int, counts):
     rt = ctypes.c_uint64()
     st = lib.hape_exchange_plan(G, rank, c, so, ro, ctypes.byref(rt))
     return st, list(so), list(ro), int(rt.value)
+
+
+def hape_join_stream(h):
+    s = ctypes.c_void_p()
+    st = lib.hape_join_stream(h, ctypes.byref(s))
+    return st, int(s.value or 0)
+
+
+def hape_debug_route(h, rel: hape_relation, is_s: int, fanout: int, out_keys: int, out_payloads: int,
+                     out_bounds: int) -> int:
+    return lib.hape_debug_route(h, ctypes.byref(rel), is_s, fanout, out_keys, out_payloads, out_bounds)
+
+
+def hape_debug_loopback_join(h, world: int, R_shards, S_shards, out, per_dest, total: hape_join_result) -> int:
+    Ra = (hape_relation * world)(*R_shards)
+    Sa = (hape_relation * world)(*S_shards)
+    return lib.hape_debug_loopback_join(h, world, Ra, Sa, ctypes.byref(out) if out is not None else None,
+                                        per_dest, ctypes.byref(total))

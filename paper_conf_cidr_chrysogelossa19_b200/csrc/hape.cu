@@ -71,11 +71,13 @@ struct hape_join {
   DevBuf recv[2];         // G>1 exchange receive buffers
   DevBuf outst[2];        // host-output staging
   DevBuf small;           // histograms, bounds, work list, counters
+  DevBuf route_ws;        // route(): per-CTA destination histograms + totals
+  DevBuf xb;              // G>1: local + gathered destination bounds
   DevBuf np_table;        // hape_nonpartitioned_join: the HBM hash table
   unsigned long long* h_res = nullptr;  // pinned: acc[4], out_ctr, (n_items | item_ctr)
   // cached CUDA graph of the local join sequence (keyed by pointers + sizes)
   cudaGraphExec_t gexec = nullptr;
-  uintptr_t gkey[14] = {};
+  uintptr_t gkey[16] = {};
   uint32_t g_launches = 0, g_join_ctas = 0;
   bool g_ev_used[HAPE_NSTAGES] = {};
   uint32_t* h_bounds = nullptr;         // pinned: gathered device-partition bounds
@@ -294,15 +296,24 @@ static uint32_t joint_grid(const hape_join* h, uint32_t nchunks) {
 
 static size_t joint_smem(uint32_t P1, uint32_t P2) { return (size_t)P1 * P2 * 2 + (size_t)P1 * 4; }
 
+// cudaFuncSetAttribute applies to the current device only: one bit per
+// device ordinal and kernel instantiation (the caller's `mask` is a static
+// of the instantiating template)
+template <class F>
+static hape_status smem_attr(hape_join* h, F kern, int bytes, uint64_t& mask) {
+  const uint64_t bit = 1ull << (h->dev & 63);
+  if (mask & bit) return HAPE_OK;
+  CK(h, cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, bytes));
+  mask |= bit;
+  return HAPE_OK;
+}
+
 template <int KW, int PW, bool AOS, bool IDENT>
 static hape_status hist_joint_t(hape_join* h, const Src& s, SegMap m, BitField bf1, BitField bf2, uint32_t P1,
                                 uint32_t P2, uint32_t* rowsum, uint16_t* part, uint32_t* ovf) {
   auto kern = k_hist_joint<KW, PW, AOS, IDENT>;
-  static bool attr_set = false;
-  if (!attr_set) {
-    CK(h, cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024));
-    attr_set = true;
-  }
+  static uint64_t attr_dev = 0;
+  CKS(smem_attr(h, kern, 200 * 1024, attr_dev));
   const uint32_t nch = m.nseg * m.cps;
   kern<<<joint_grid(h, nch), HJ_THREADS, joint_smem(P1, P2), h->stream>>>(s.in, m, P1, P2, rowsum, part,
                                                                         ovf);
@@ -359,12 +370,8 @@ template <int KW, int PW, bool AOS, class C, bool IDENT, bool CLAIM>
 static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* offs,
                              void* out) {
   const size_t smem = ScLayout<KW, PW, AOS, C>::bytes(P);
-  static bool attr_set = false;
-  if (!attr_set) {
-    CK(h, cudaFuncSetAttribute(k_scatter<KW, PW, AOS, C, IDENT, CLAIM>, cudaFuncAttributeMaxDynamicSharedMemorySize,
-                               220 * 1024));
-    attr_set = true;
-  }
+  static uint64_t attr_dev = 0;
+  CKS(smem_attr(h, k_scatter<KW, PW, AOS, C, IDENT, CLAIM>, 220 * 1024, attr_dev));
   const unsigned grid = m.nseg * m.cps;
   if (grid == 0) return HAPE_OK;
   k_scatter<KW, PW, AOS, C, IDENT, CLAIM><<<grid, C::NT, smem, h->stream>>>(s.in, m, bf, P, offs,
@@ -439,11 +446,8 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
   static const int nrb_env = env_int("HAPE_JN_NRB", 0), nsb_env = env_int("HAPE_JN_NSB", 0);
   a.nsb = SR ? (uint32_t)std::min(8, std::max(2, nsb_env ? nsb_env : (SU >= 4 ? 3 : 2))) : 0u;
   a.nrb = SR ? (uint32_t)std::min(2, std::max(1, nrb_env ? nrb_env : 2)) : 2u;
-  static bool attr_set = false;
-  if (!attr_set) {
-    CK(h, cudaFuncSetAttribute(kern, cudaFuncAttributeMaxDynamicSharedMemorySize, 200 * 1024));
-    attr_set = true;
-  }
+  static uint64_t attr_dev = 0;
+  CKS(smem_attr(h, kern, 200 * 1024, attr_dev));
   auto occ = [&](uint32_t sb, uint32_t nrb, int* per_sm) -> hape_status {
     const size_t smem = join_smem_bytes<KW, PRW, PSW, SU, NC>(a.cap, sb, nrb, a.nsb);
     *per_sm = 0;
@@ -742,63 +746,60 @@ extern "C" hape_status hape_exchange_plan(int world_size, int rank, const uint64
   return HAPE_OK;
 }
 
-static hape_status exchange(hape_join* h, Src in[2], Src out[2]) {
-  const int G = std::max(1, h->cfg.world_size), me = h->cfg.rank;
+// a2-a4: device partition of one relation by destination = the top log2(G)
+// bits of h (R14) -- hist -> scan -> smem-staged scatter with
+// fan-out G -- into `out` (AoS tuples, destination-major) and bounds[G+1]
+// (device, tuple offsets relative to `out`).  The router of P643-652 ("hash-
+// based" policy) as one partitioning pass.
+static hape_status route(hape_join* h, const Src& in, uint32_t G, void* out, uint32_t* bounds) {
   const int kw = key_width(h->cfg);
   const uint32_t g = ceil_log2_u64((uint64_t)G);
   const uint32_t HW = kw * 8;
-  const BitField bf{g ? HW - g : 0u, (uint32_t)G - 1};  // destination = top g bits of h (R14)
-  // layout in small: per side hist[G*cps], rowsum[G], and the local bounds block [2][G+1] + gathered [G][2][G+1]
-  Carve cv;
-  uint32_t cps[2];
-  size_t hist_off[2], rs_off[2];
-  for (int s = 0; s < 2; s++) {
-    cps[s] = cps_for(h, in[s].n, 1);
-    hist_off[s] = cv.take((size_t)G * cps[s] * 4);
-    rs_off[s] = cv.take((size_t)G * 4);
-  }
-  const size_t bl_off = cv.take((size_t)2 * (G + 1) * 4);
-  const size_t bg_off = cv.take((size_t)G * 2 * (G + 1) * 4);
-  CKS(ensure(h, h->small, cv.off));
-  CK(h, cudaMemsetAsync(at<char>(h, rs_off[0]), 0, (size_t)G * 4, h->stream));
-  CK(h, cudaMemsetAsync(at<char>(h, rs_off[1]), 0, (size_t)G * 4, h->stream));
+  const BitField bf{g ? HW - g : 0u, G - 1};
+  const uint32_t cps = cps_for(h, in.n, 1);
+  const size_t hist_b = ((size_t)G * cps * 4 + 255) & ~(size_t)255;
+  CKS(ensure(h, h->route_ws, hist_b + (size_t)G * 4));
+  uint32_t* hist = static_cast<uint32_t*>(h->route_ws.p);
+  uint32_t* rs = hist + hist_b / 4;
+  CK(h, cudaMemsetAsync(rs, 0, (size_t)G * 4, h->stream));
+  const SegMap m{nullptr, 1u, cps, in.n};
+  CKS(launch_hist(h, kw, in, m, bf, G, hist, rs));
+  CKS(launch_scan(h, m, G, hist, rs, bounds));
+  CKS(launch_scatter(h, kw, in, m, bf, G, hist, out));
+  return HAPE_OK;
+}
+
+static hape_status exchange(hape_join* h, Src in[2], Src out[2]) {
+  const int G = std::max(1, h->cfg.world_size), me = h->cfg.rank;
+  const int kw = key_width(h->cfg);
+  // bounds: local [2][G+1], then gathered [G][2][G+1]
+  const size_t nl = (size_t)2 * (G + 1), nb = (size_t)G * nl;
+  CKS(ensure(h, h->xb, (nl + nb) * 4));
+  uint32_t* bl = static_cast<uint32_t*>(h->xb.p);
+  uint32_t* bg = bl + nl;
   mark(h, HAPE_STAGE_DEVPART);
   size_t tb[2];
   for (int s = 0; s < 2; s++) {
     tb[s] = tup_bytes(kw, in[s].pw);
     CKS(ensure(h, h->send[s], (size_t)in[s].n * tb[s] + 16));
-    SegMap m{nullptr, 1u, cps[s], in[s].n};
-    uint32_t* hist = at<uint32_t>(h, hist_off[s]);
-    uint32_t* rs = at<uint32_t>(h, rs_off[s]);
-    uint32_t* bl = at<uint32_t>(h, bl_off) + s * (G + 1);
-    CKS(launch_hist(h, kw, in[s], m, bf, (uint32_t)G, hist, rs));
-    CKS(launch_scan(h, m, (uint32_t)G, hist, rs, bl));
-    CKS(launch_scatter(h, kw, in[s], m, bf, (uint32_t)G, hist, h->send[s].p));
+    CKS(route(h, in[s], (uint32_t)G, h->send[s].p, bl + s * (G + 1)));
   }
   mark(h, HAPE_STAGE_EXCHANGE);
   // count exchange: all-gather every rank's destination bounds
-  CKN(h, ncclAllGather(at<uint32_t>(h, bl_off), at<uint32_t>(h, bg_off), (size_t)2 * (G + 1), ncclUint32, h->comm,
-                       h->stream));
-  const size_t nb = (size_t)G * 2 * (G + 1);
+  CKN(h, ncclAllGather(bl, bg, nl, ncclUint32, h->comm, h->stream));
   if (h->h_bounds_cap < nb) {
     if (h->h_bounds) cudaFreeHost(h->h_bounds);
-  for (auto& p : h->hp)
-    if (p) cudaFreeHost(p);
-  for (auto& set : h->cpst)
-    for (auto& b : set)
-      if (b.p) cudaFree(b.p);
-  for (auto& pr : h->ev_h2d)
-    for (auto& e : pr)
-      if (e) cudaEventDestroy(e);
+    h->h_bounds = nullptr;
+    h->h_bounds_cap = 0;
     CK(h, cudaMallocHost(&h->h_bounds, nb * 4));
     h->h_bounds_cap = nb;
   }
-  CK(h, cudaMemcpyAsync(h->h_bounds, at<uint32_t>(h, bg_off), nb * 4, cudaMemcpyDeviceToHost, h->stream));
+  CK(h, cudaMemcpyAsync(h->h_bounds, bg, nb * 4, cudaMemcpyDeviceToHost, h->stream));
   CK(h, cudaStreamSynchronize(h->stream));
   for (int s = 0; s < 2; s++) {
     std::vector<uint64_t> counts((size_t)G * G), soff(G), roff(G);
     for (int src = 0; src < G; src++) {
-      const uint32_t* b = h->h_bounds + (size_t)src * 2 * (G + 1) + s * (G + 1);
+      const uint32_t* b = h->h_bounds + (size_t)src * nl + s * (G + 1);
       for (int d = 0; d < G; d++) counts[(size_t)src * G + d] = b[d + 1] - b[d];
     }
     uint64_t rtot = 0;
@@ -839,43 +840,24 @@ static void stage_times(hape_join* h, hape_join_result* res) {
 }
 
 // ---------------------------------------------------------------------------
-// the join
+// the local join (a6-a13 over one GPU's share): plan, radix passes, work
+// list, build+probe, local result D2H into h_res[0..5] (acc[4], out_ctr,
+// ctrs).  Enqueued on h->stream; no host sync.  When every pointer and size
+// matches the previous call the sequence is replayed as one captured CUDA
+// graph (launch-latency bound small joins, BASELINE configs[0]).
 // ---------------------------------------------------------------------------
-static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_relation* S, const hape_output* out,
-                             hape_join_result* res) {
+struct MatOut {
+  bool on = false;
+  void* r = nullptr;
+  void* s = nullptr;
+  uint64_t cap = 0;
+};
+
+static hape_status local_join(hape_join* h, const Src loc_in[2], const MatOut& mo, cudaEvent_t side1_ready,
+                              bool graphable, hape_plan* pl_out) {
   const hape_join_config& c = h->cfg;
   const int kw = key_width(c), prw = pay_width(c.r_payload_type), psw = pay_width(c.s_payload_type);
-  CKS(check_rel(h, R, kw, prw, "R"));
-  CKS(check_rel(h, S, kw, psw, "S"));
-  const bool mat = out && out->capacity > 0;
-  if (mat) {
-    if (!out->r_payload || !out->s_payload) return fail(h, HAPE_ERR_INVALID_ARG, "output buffers NULL");
-    if (out->mem != HAPE_MEM_DEVICE && out->mem != HAPE_MEM_HOST) return fail(h, HAPE_ERR_INVALID_ARG, "out.mem");
-  }
-  CK(h, cudaSetDevice(h->dev));
-  memset(res, 0, sizeof *res);
-  for (int i = 0; i < HAPE_NSTAGES; i++) h->ev_used[i] = false;
-  h->launches = 0;
-  const int world = c.world_size > 1 ? c.world_size : 1;
-
-  mark(h, HAPE_STAGE_TOTAL);
-  mark(h, HAPE_STAGE_H2D);
-  Src in[2];
-  // host-resident S (single GPU): copy it on the copy stream, overlapping the
-  // R copy's successors (R's radix passes run while S is in flight)
-  const bool overlap = world == 1 && !h->comm && S->mem == HAPE_MEM_HOST && S->n > 0;
-  CKS(stage_in(h, R, kw, prw, h->stage[0], h->stage[1], &in[0]));
-  if (overlap) {
-    CK(h, cudaEventRecord(h->ev_copy, h->stream));          // S staging buffers are free
-    CK(h, cudaStreamWaitEvent(h->copy_stream, h->ev_copy, 0));
-    CKS(stage_in(h, S, kw, psw, h->stage[2], h->stage[3], &in[1], h->copy_stream));
-    CK(h, cudaEventRecord(h->ev_copy, h->copy_stream));
-  } else {
-    CKS(stage_in(h, S, kw, psw, h->stage[2], h->stage[3], &in[1]));
-  }
-  Src loc[2] = {in[0], in[1]};
-  if (world > 1 || h->comm) CKS(exchange(h, in, loc));
-
+  const Src loc[2] = {loc_in[0], loc_in[1]};
   hape_plan pl;
   if (make_plan(h, loc[0].n, loc[1].n, &pl) != HAPE_OK)
     return fail(h, HAPE_ERR_INVALID_ARG, "invalid radix plan (bits/passes)");
@@ -887,21 +869,6 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
     CKS(ensure(h, h->ping[s], n_loc[s] * tup_bytes(kw, pw[s]) + 16));
     if (pl.passes == 2) CKS(ensure(h, h->pong[s], n_loc[s] * tup_bytes(kw, pw[s]) + 16));
   }
-  void* mat_r = nullptr;
-  void* mat_s = nullptr;
-  if (mat) {
-    mat_r = out->r_payload;
-    mat_s = out->s_payload;
-    if (out->mem == HAPE_MEM_HOST) {
-      CKS(ensure(h, h->outst[0], out->capacity * prw));
-      CKS(ensure(h, h->outst[1], out->capacity * psw));
-      mat_r = h->outst[0].p;
-      mat_s = h->outst[1].p;
-    }
-  }
-  // the device-side sequence of one local join; replayed as one CUDA graph
-  // when every pointer and size matches the previous call (launch-latency
-  // bound small joins, BASELINE configs[0])
   const uint32_t Q = 1u << (pl.bits[0] + (pl.passes == 2 ? pl.bits[1] : 0));
   uint32_t* ctrs = at<uint32_t>(h, L.ctrs);  // [0] n_items
   auto enqueue = [&]() -> hape_status {
@@ -910,7 +877,7 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
     for (int s = 0; s < 2; s++) io[s] = PassIO{loc[s], h->ping[s].p, h->pong[s].p};
     const void* ft[2];
     const uint32_t* fb[2];
-    CKS(run_partition_stages(h, pl, L, io, 2, ft, fb, overlap ? h->ev_copy : nullptr));
+    CKS(run_partition_stages(h, pl, L, io, 2, ft, fb, side1_ready));
     mark(h, HAPE_STAGE_WORKLIST);
     k_worklist<<<(Q + WL_THREADS - 1) / WL_THREADS, WL_THREADS, 0, h->stream>>>(fb[0], fb[1], Q, pl.probe_slice,
                                                                                 at<uint2>(h, L.items), ctrs);
@@ -922,7 +889,7 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
     ja.items = at<uint2>(h, L.items); ja.n_items = ctrs;
     ja.cap = pl.build_cap; ja.slice = pl.probe_slice; ja.slot_bits = pl.slot_bits;
     ja.acc = at<unsigned long long>(h, L.acc);
-    ja.out_r = mat_r; ja.out_s = mat_s; ja.out_cap = mat ? out->capacity : 0;
+    ja.out_r = mo.r; ja.out_s = mo.s; ja.out_cap = mo.on ? mo.cap : 0;
     ja.out_ctr = at<unsigned long long>(h, L.out_ctr);
     static const uint32_t jn_dbg = [] { const char* e = getenv("HAPE_JN_DBG"); return e ? (uint32_t)atoi(e) : 0u; }();
     ja.dbg = jn_dbg;  // timing experiments only: results are wrong when set
@@ -931,7 +898,7 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
     // larger slices would thrash L2 a stage ahead of their use)
     static const int pf_env = [] { const char* e = getenv("HAPE_JN_PF"); return e ? atoi(e) : -1; }();
     ja.pf_bytes = pf_env >= 0 ? (uint32_t)pf_env : 32768u;
-    CKS(launch_join(h, kw, prw, psw, ja, mat, &pl.join_ctas));
+    CKS(launch_join(h, kw, prw, psw, ja, mo.on, &pl.join_ctas));
     mark(h, HAPE_STAGE_FINALIZE);
     // local result: acc[4], out_ctr, ctrs
     CK(h, cudaMemcpyAsync(h->h_res, at<char>(h, L.acc), 4 * 8, cudaMemcpyDeviceToHost, h->stream));
@@ -940,13 +907,13 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
     return HAPE_OK;
   };
   static const bool no_graph = getenv("HAPE_NO_GRAPH") != nullptr;
-  const bool graphable = !no_graph && !h->in_coprocess && world == 1 && !h->comm && R->mem == HAPE_MEM_DEVICE &&
-                         S->mem == HAPE_MEM_DEVICE && (!mat || out->mem == HAPE_MEM_DEVICE);
-  if (graphable) {
-    const uintptr_t key[] = {(uintptr_t)R->key, (uintptr_t)R->payload, (uintptr_t)R->n, (uintptr_t)S->key,
-                             (uintptr_t)S->payload, (uintptr_t)S->n, (uintptr_t)mat_r, (uintptr_t)mat_s,
-                             (uintptr_t)(mat ? out->capacity : 0), (uintptr_t)h->small.p, (uintptr_t)h->ping[0].p,
-                             (uintptr_t)h->ping[1].p, (uintptr_t)h->pong[0].p, (uintptr_t)h->pong[1].p};
+  if (graphable && !no_graph && !side1_ready) {
+    const uintptr_t key[] = {(uintptr_t)loc[0].in.k, (uintptr_t)loc[0].in.p, (uintptr_t)loc[0].in.t,
+                             (uintptr_t)loc[0].n,    (uintptr_t)loc[1].in.k, (uintptr_t)loc[1].in.p,
+                             (uintptr_t)loc[1].in.t, (uintptr_t)loc[1].n,    (uintptr_t)mo.r,
+                             (uintptr_t)mo.s,        (uintptr_t)(mo.on ? mo.cap : 0), (uintptr_t)h->small.p,
+                             (uintptr_t)h->ping[0].p, (uintptr_t)h->ping[1].p, (uintptr_t)h->pong[0].p,
+                             (uintptr_t)h->pong[1].p};
     static_assert(sizeof key == sizeof h->gkey, "graph key size");
     if (!h->gexec || memcmp(key, h->gkey, sizeof key) != 0) {
       if (h->gexec) { cudaGraphExecDestroy(h->gexec); h->gexec = nullptr; }
@@ -971,9 +938,89 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   } else {
     CKS(enqueue());
   }
+  *pl_out = pl;
+  return HAPE_OK;
+}
+
+static hape_status check_out(hape_join* h, const hape_output* out) {
+  if (!out || out->capacity == 0) return HAPE_OK;
+  if (!out->r_payload || !out->s_payload) return fail(h, HAPE_ERR_INVALID_ARG, "output buffers NULL");
+  if (out->mem != HAPE_MEM_DEVICE && out->mem != HAPE_MEM_HOST) return fail(h, HAPE_ERR_INVALID_ARG, "out.mem");
+  return HAPE_OK;
+}
+
+// device targets of the pair output: the caller's buffers, or handle-owned
+// staging for host-resident outputs (copied back after the join)
+static hape_status mat_targets(hape_join* h, const hape_output* out, MatOut* mo) {
+  *mo = MatOut{};
+  if (!out || out->capacity == 0) return HAPE_OK;
+  mo->on = true;
+  mo->cap = out->capacity;
+  mo->r = out->r_payload;
+  mo->s = out->s_payload;
+  if (out->mem == HAPE_MEM_HOST) {
+    CKS(ensure(h, h->outst[0], out->capacity * pay_width(h->cfg.r_payload_type)));
+    CKS(ensure(h, h->outst[1], out->capacity * pay_width(h->cfg.s_payload_type)));
+    mo->r = h->outst[0].p;
+    mo->s = h->outst[1].p;
+  }
+  return HAPE_OK;
+}
+
+static void fill_plan_fields(hape_join_result* res, const hape_plan& pl, uint64_t nr, uint64_t ns) {
+  res->r_local = nr;
+  res->s_local = ns;
+  res->passes = pl.passes;
+  res->bits[0] = pl.bits[0];
+  res->bits[1] = pl.passes == 2 ? pl.bits[1] : 0;
+  res->n_partitions = 1u << (pl.bits[0] + (pl.passes == 2 ? pl.bits[1] : 0));
+}
+
+// ---------------------------------------------------------------------------
+// the join
+// ---------------------------------------------------------------------------
+static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_relation* S, const hape_output* out,
+                             hape_join_result* res) {
+  const hape_join_config& c = h->cfg;
+  const int kw = key_width(c), prw = pay_width(c.r_payload_type), psw = pay_width(c.s_payload_type);
+  CKS(check_rel(h, R, kw, prw, "R"));
+  CKS(check_rel(h, S, kw, psw, "S"));
+  CKS(check_out(h, out));
+  const bool mat = out && out->capacity > 0;
+  CK(h, cudaSetDevice(h->dev));
+  memset(res, 0, sizeof *res);
+  for (int i = 0; i < HAPE_NSTAGES; i++) h->ev_used[i] = false;
+  h->launches = 0;
+  const int world = c.world_size > 1 ? c.world_size : 1;
+
+  mark(h, HAPE_STAGE_TOTAL);
+  mark(h, HAPE_STAGE_H2D);
+  Src in[2];
+  // host-resident S (single GPU): copy it on the copy stream, overlapping the
+  // R copy's successors (R's radix passes run while S is in flight)
+  const bool overlap = world == 1 && !h->comm && S->mem == HAPE_MEM_HOST && S->n > 0;
+  CKS(stage_in(h, R, kw, prw, h->stage[0], h->stage[1], &in[0]));
+  if (overlap) {
+    CK(h, cudaEventRecord(h->ev_copy, h->stream));          // S staging buffers are free
+    CK(h, cudaStreamWaitEvent(h->copy_stream, h->ev_copy, 0));
+    CKS(stage_in(h, S, kw, psw, h->stage[2], h->stage[3], &in[1], h->copy_stream));
+    CK(h, cudaEventRecord(h->ev_copy, h->copy_stream));
+  } else {
+    CKS(stage_in(h, S, kw, psw, h->stage[2], h->stage[3], &in[1]));
+  }
+  Src loc[2] = {in[0], in[1]};
+  if (world > 1 || h->comm) CKS(exchange(h, in, loc));
+
+  MatOut mo;
+  CKS(mat_targets(h, out, &mo));
+  const bool graphable = !h->in_coprocess && world == 1 && !h->comm && R->mem == HAPE_MEM_DEVICE &&
+                         S->mem == HAPE_MEM_DEVICE && (!mat || out->mem == HAPE_MEM_DEVICE);
+  hape_plan pl;
+  CKS(local_join(h, loc, mo, overlap ? h->ev_copy : nullptr, graphable, &pl));
   if (world > 1 || h->comm) {
     // global result: NCCL allreduce (sum, u64, wrapping) of the four fields
-    unsigned long long* acc = at<unsigned long long>(h, L.acc);
+    // (layout_for puts acc[4] first in the small buffer)
+    unsigned long long* acc = at<unsigned long long>(h, 0);
     CKN(h, ncclAllReduce(acc, acc, 4, ncclUint64, ncclSum, h->comm, h->stream));
     CK(h, cudaMemcpyAsync(h->h_res + 6, acc, 4 * 8, cudaMemcpyDeviceToHost, h->stream));
   }
@@ -991,15 +1038,10 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   res->n_required = r[0];
   res->n_written = mat ? std::min<uint64_t>(r[4], out->capacity) : 0;
   res->n_items = (uint32_t)(r[5] & 0xFFFFFFFFu);
-  res->r_local = loc[0].n;
-  res->s_local = loc[1].n;
-  res->passes = pl.passes;
-  res->bits[0] = pl.bits[0];
-  res->bits[1] = pl.passes == 2 ? pl.bits[1] : 0;
-  res->n_partitions = Q;
+  fill_plan_fields(res, pl, loc[0].n, loc[1].n);
   if (mat && out->mem == HAPE_MEM_HOST && res->n_written) {
-    CK(h, cudaMemcpyAsync(out->r_payload, mat_r, res->n_written * prw, cudaMemcpyDeviceToHost, h->stream));
-    CK(h, cudaMemcpyAsync(out->s_payload, mat_s, res->n_written * psw, cudaMemcpyDeviceToHost, h->stream));
+    CK(h, cudaMemcpyAsync(out->r_payload, mo.r, res->n_written * prw, cudaMemcpyDeviceToHost, h->stream));
+    CK(h, cudaMemcpyAsync(out->s_payload, mo.s, res->n_written * psw, cudaMemcpyDeviceToHost, h->stream));
   }
   cudaEventRecord(h->ev[HAPE_NSTAGES], h->stream);
   CK(h, cudaStreamSynchronize(h->stream));
@@ -1008,6 +1050,152 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   if (mat && r[4] > out->capacity)
     return fail(h, HAPE_ERR_OUTPUT_CAPACITY, "join produced %llu pairs > capacity %llu", (unsigned long long)r[4],
                 (unsigned long long)out->capacity);
+  return HAPE_OK;
+}
+
+// ---------------------------------------------------------------------------
+// G simulated ranks on this one GPU (hape_debug_loopback_join): every
+// device step of the G>1 path -- route() of each source shard with fan-out
+// G, the count matrix, hape_exchange_plan's offsets, the AoS receive layout
+// and the local join of each destination's received tuples -- with the NCCL
+// transport replaced by device-to-device copies of the same segments to the
+// same receive offsets.
+// ---------------------------------------------------------------------------
+static hape_status loopback_impl(hape_join* h, int G, const hape_relation* Rs, const hape_relation* Ss,
+                                 const hape_output* out, hape_join_result* per_dest, hape_join_result* total) {
+  const hape_join_config& c = h->cfg;
+  const int kw = key_width(c), prw = pay_width(c.r_payload_type), psw = pay_width(c.s_payload_type);
+  if (G < 1 || G > 64 || (G & (G - 1))) return fail(h, HAPE_ERR_INVALID_ARG, "world must be a power of two <= 64");
+  if (!Rs || !Ss || !total) return fail(h, HAPE_ERR_INVALID_ARG, "NULL shard arrays or result");
+  if (c.world_size > 1 || h->comm) return fail(h, HAPE_ERR_UNSUPPORTED, "loopback needs a single-GPU handle");
+  CKS(check_out(h, out));
+  const int pws[2] = {prw, psw};
+  const hape_relation* shards[2] = {Rs, Ss};
+  uint64_t ntot[2] = {0, 0};
+  for (int s = 0; s < 2; s++)
+    for (int i = 0; i < G; i++) {
+      CKS(check_rel(h, &shards[s][i], kw, pws[s], s ? "S shard" : "R shard"));
+      if (shards[s][i].mem != HAPE_MEM_DEVICE)
+        return fail(h, HAPE_ERR_UNSUPPORTED, "loopback shards must be device-resident");
+      ntot[s] += shards[s][i].n;
+    }
+  if (ntot[0] >= 0xFFFFFFFFull || ntot[1] >= 0xFFFFFFFFull)
+    return fail(h, HAPE_ERR_UNSUPPORTED, "loopback total >= 2^32 tuples");
+  CK(h, cudaSetDevice(h->dev));
+  memset(total, 0, sizeof *total);
+  for (int i = 0; i < HAPE_NSTAGES; i++) h->ev_used[i] = false;
+  h->launches = 0;
+  // (a2-a4) route every source shard into its region of the send buffer
+  size_t tb[2];
+  for (int s = 0; s < 2; s++) {
+    tb[s] = tup_bytes(kw, pws[s]);
+    CKS(ensure(h, h->send[s], ntot[s] * tb[s] + 16));
+  }
+  CKS(ensure(h, h->xb, (size_t)2 * G * (G + 1) * 4));
+  uint32_t* dbounds = static_cast<uint32_t*>(h->xb.p);
+  std::vector<uint64_t> base[2];
+  for (int s = 0; s < 2; s++) {
+    base[s].assign(G + 1, 0);
+    for (int i = 0; i < G; i++) {
+      Src in;
+      CKS(stage_in(h, &shards[s][i], kw, pws[s], h->stage[0], h->stage[1], &in));
+      CKS(route(h, in, (uint32_t)G, static_cast<char*>(h->send[s].p) + base[s][i] * tb[s],
+                dbounds + ((size_t)s * G + i) * (G + 1)));
+      base[s][i + 1] = base[s][i] + shards[s][i].n;
+    }
+  }
+  // (a5) count exchange
+  std::vector<uint32_t> hb((size_t)2 * G * (G + 1));
+  CK(h, cudaMemcpyAsync(hb.data(), dbounds, hb.size() * 4, cudaMemcpyDeviceToHost, h->stream));
+  CK(h, cudaStreamSynchronize(h->stream));
+  std::vector<uint64_t> counts[2];
+  for (int s = 0; s < 2; s++) {
+    counts[s].assign((size_t)G * G, 0);
+    for (int src = 0; src < G; src++) {
+      const uint32_t* b = hb.data() + ((size_t)s * G + src) * (G + 1);
+      for (int d = 0; d < G; d++) counts[s][(size_t)src * G + d] = b[d + 1] - b[d];
+    }
+  }
+  MatOut mo0;
+  CKS(mat_targets(h, out, &mo0));
+  uint64_t written = 0, required = 0;
+  bool over = false;
+  for (int d = 0; d < G; d++) {
+    Src loc[2];
+    for (int s = 0; s < 2; s++) {
+      std::vector<uint64_t> soff(G), roff(G);
+      uint64_t rtot = 0;
+      hape_exchange_plan(G, d, counts[s].data(), soff.data(), roff.data(), &rtot);
+      CKS(ensure(h, h->recv[s], rtot * tb[s] + 16));
+      // the all-to-allv: source src's destination-d segment -> roff[src]
+      for (int src = 0; src < G; src++) {
+        const uint64_t cnt = counts[s][(size_t)src * G + d];
+        if (!cnt) continue;
+        const uint32_t* b = hb.data() + ((size_t)s * G + src) * (G + 1);
+        CK(h, cudaMemcpyAsync(static_cast<char*>(h->recv[s].p) + roff[src] * tb[s],
+                              static_cast<const char*>(h->send[s].p) + (base[s][src] + b[d]) * tb[s], cnt * tb[s],
+                              cudaMemcpyDeviceToDevice, h->stream));
+      }
+      loc[s] = Src{PartIn{nullptr, nullptr, h->recv[s].p}, true, (uint32_t)rtot, pws[s]};
+    }
+    MatOut mo = mo0;
+    if (mo.on) {
+      const uint64_t off = std::min(written, mo.cap);
+      mo.cap -= off;
+      mo.r = static_cast<char*>(mo.r) + off * prw;
+      mo.s = static_cast<char*>(mo.s) + off * psw;
+      mo.on = mo.cap > 0;
+    }
+    hape_plan pl;
+    CKS(local_join(h, loc, mo, nullptr, false, &pl));
+    CK(h, cudaStreamSynchronize(h->stream));
+    const unsigned long long* r = h->h_res;
+    const uint64_t nw = mo.on ? std::min<uint64_t>(r[4], mo.cap) : 0;
+    if (per_dest) {
+      hape_join_result& pd = per_dest[d];
+      memset(&pd, 0, sizeof pd);
+      pd.local_match_count = r[0];
+      pd.local_sum_r = r[1];
+      pd.local_sum_s = r[2];
+      pd.local_pair_checksum = r[3];
+      pd.n_required = r[0];
+      pd.n_written = nw;
+      pd.n_items = (uint32_t)(r[5] & 0xFFFFFFFFu);
+      fill_plan_fields(&pd, pl, loc[0].n, loc[1].n);
+    }
+    total->match_count += r[0];
+    total->sum_r_payload += r[1];
+    total->sum_s_payload += r[2];
+    total->pair_checksum += r[3];
+    written += nw;
+    required += r[0];
+    if (mo0.on && r[0] > nw) over = true;
+  }
+  total->local_match_count = total->match_count;
+  total->local_sum_r = total->sum_r_payload;
+  total->local_sum_s = total->sum_s_payload;
+  total->local_pair_checksum = total->pair_checksum;
+  total->n_written = written;
+  total->n_required = required;
+  total->r_local = ntot[0];
+  total->s_local = ntot[1];
+  total->n_partitions = (uint32_t)G;
+  total->kernel_launches = h->launches;
+  if (per_dest)
+    for (int d = 0; d < G; d++) {
+      per_dest[d].match_count = total->match_count;
+      per_dest[d].sum_r_payload = total->sum_r_payload;
+      per_dest[d].sum_s_payload = total->sum_s_payload;
+      per_dest[d].pair_checksum = total->pair_checksum;
+    }
+  if (mo0.on && written && out->mem == HAPE_MEM_HOST) {
+    CK(h, cudaMemcpyAsync(out->r_payload, mo0.r, written * prw, cudaMemcpyDeviceToHost, h->stream));
+    CK(h, cudaMemcpyAsync(out->s_payload, mo0.s, written * psw, cudaMemcpyDeviceToHost, h->stream));
+    CK(h, cudaStreamSynchronize(h->stream));
+  }
+  if (over)
+    return fail(h, HAPE_ERR_OUTPUT_CAPACITY, "loopback join produced %llu pairs > capacity %llu",
+                (unsigned long long)required, (unsigned long long)out->capacity);
   return HAPE_OK;
 }
 
@@ -1250,6 +1438,8 @@ hape_status hape_join_destroy(hape_join* h) {
     if (b.p) cudaFree(b.p);
   if (h->gexec) cudaGraphExecDestroy(h->gexec);
   if (h->small.p) cudaFree(h->small.p);
+  if (h->route_ws.p) cudaFree(h->route_ws.p);
+  if (h->xb.p) cudaFree(h->xb.p);
   if (h->np_table.p) cudaFree(h->np_table.p);
   if (h->h_res) cudaFreeHost(h->h_res);
   if (h->h_bounds) cudaFreeHost(h->h_bounds);
@@ -1333,6 +1523,50 @@ hape_status hape_debug_partition(hape_join* h, const hape_relation* rel, int is_
   CK(h, cudaStreamSynchronize(h->stream));
   if (plan_out) *plan_out = pl;
   return HAPE_OK;
+}
+
+hape_status hape_join_stream(const hape_join* h, void** out_stream) {
+  if (!h || !out_stream) return HAPE_ERR_INVALID_ARG;
+  *out_stream = h->stream;
+  return HAPE_OK;
+}
+
+hape_status hape_debug_route(hape_join* h, const hape_relation* rel, int is_s, int fanout, void* out_keys,
+                             void* out_payloads, uint32_t* out_bounds) {
+  if (!h) return HAPE_ERR_INVALID_ARG;
+  try {
+    const hape_join_config& c = h->cfg;
+    const int kw = key_width(c), pw = pay_width(is_s ? c.s_payload_type : c.r_payload_type);
+    CKS(check_rel(h, rel, kw, pw, "rel"));
+    if (fanout < 1 || fanout > 4096 || (fanout & (fanout - 1)))
+      return fail(h, HAPE_ERR_INVALID_ARG, "fanout must be a power of two in [1, 4096]");
+    if (rel->n && (!out_keys || !out_payloads)) return fail(h, HAPE_ERR_INVALID_ARG, "outputs NULL");
+    if (!out_bounds) return fail(h, HAPE_ERR_INVALID_ARG, "out_bounds NULL");
+    CK(h, cudaSetDevice(h->dev));
+    h->launches = 0;
+    Src in;
+    CKS(stage_in(h, rel, kw, pw, h->stage[0], h->stage[1], &in));
+    CKS(ensure(h, h->send[0], rel->n * tup_bytes(kw, pw) + 16));
+    CKS(ensure(h, h->xb, ((size_t)fanout + 1) * 4));
+    CKS(route(h, in, (uint32_t)fanout, h->send[0].p, static_cast<uint32_t*>(h->xb.p)));
+    CKS(launch_unpack(h, kw, pw, h->send[0].p, (uint32_t)rel->n, out_keys, out_payloads));
+    CK(h, cudaMemcpyAsync(out_bounds, h->xb.p, ((size_t)fanout + 1) * 4, cudaMemcpyDeviceToDevice, h->stream));
+    CK(h, cudaStreamSynchronize(h->stream));
+    return HAPE_OK;
+  } catch (...) {
+    return fail(h, HAPE_ERR_CUDA, "unexpected C++ exception");
+  }
+}
+
+hape_status hape_debug_loopback_join(hape_join* h, int world, const hape_relation* R_shards,
+                                     const hape_relation* S_shards, const hape_output* out,
+                                     hape_join_result* per_dest, hape_join_result* total) {
+  if (!h) return HAPE_ERR_INVALID_ARG;
+  try {
+    return loopback_impl(h, world, R_shards, S_shards, out, per_dest, total);
+  } catch (...) {
+    return fail(h, HAPE_ERR_CUDA, "unexpected C++ exception");
+  }
 }
 
 hape_status hape_nccl_unique_id(void* out_id_128) {

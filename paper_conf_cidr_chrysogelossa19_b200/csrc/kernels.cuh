@@ -1271,19 +1271,26 @@ k_build_probe(JoinArgs a) {
           jn_probe_batch<KW, PRW, PSW, MAT, JN_U, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
           base += BATCH;
         }
-        const uint32_t rem = st.s_hi > base ? st.s_hi - base : 0;
-        if (rem > 2 * JN_CONSUMERS) {
-          Tup<KW, PSW> x[4];
-          jn_load_batch<KW, PSW, 4, JN_CONSUMERS>(a, base, st.s_hi, x);
-          jn_probe_batch<KW, PRW, PSW, MAT, 4, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
-        } else if (rem > JN_CONSUMERS) {
-          Tup<KW, PSW> x[2];
-          jn_load_batch<KW, PSW, 2, JN_CONSUMERS>(a, base, st.s_hi, x);
-          jn_probe_batch<KW, PRW, PSW, MAT, 2, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
-        } else if (rem > 0) {
-          Tup<KW, PSW> x[1];
-          jn_load_batch<KW, PSW, 1, JN_CONSUMERS>(a, base, st.s_hi, x);
-          jn_probe_batch<KW, PRW, PSW, MAT, 1, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+        // ragged tail (< BATCH tuples, any JN_U): 4-, 2- and 1-wide batches
+        // until the slice is exhausted (rem is uniform over the consumers)
+        while (st.s_hi > base) {
+          const uint32_t rem = st.s_hi - base;
+          if (rem > 2 * JN_CONSUMERS) {
+            Tup<KW, PSW> x[4];
+            jn_load_batch<KW, PSW, 4, JN_CONSUMERS>(a, base, st.s_hi, x);
+            jn_probe_batch<KW, PRW, PSW, MAT, 4, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+            base += 4 * JN_CONSUMERS;
+          } else if (rem > JN_CONSUMERS) {
+            Tup<KW, PSW> x[2];
+            jn_load_batch<KW, PSW, 2, JN_CONSUMERS>(a, base, st.s_hi, x);
+            jn_probe_batch<KW, PRW, PSW, MAT, 2, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+            base += 2 * JN_CONSUMERS;
+          } else {
+            Tup<KW, PSW> x[1];
+            jn_load_batch<KW, PSW, 1, JN_CONSUMERS>(a, base, st.s_hi, x);
+            jn_probe_batch<KW, PRW, PSW, MAT, 1, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+            base += JN_CONSUMERS;
+          }
         }
       }
       consumer_sync<JN_CONSUMERS>();  // everyone is done with heads/next and ring buffer bi

@@ -31,9 +31,10 @@ def test_reference_arm_json_line():
 
 
 def test_reference_arm_multirank():
-    # rank 0 of a 2-rank launch prints the c4 (strong-scaling) line; rank 1 exits silently
+    # rank 0 of a 2-rank launch prints the line of the same c2 workload as N=1
+    # (weak scaling at every N); rank 1 exits silently
     lines = _run({"WORLD_SIZE": "2", "RANK": "0"}, "--gpus", "2", "--steps", "1", "--warmup", "1",
                  "--ref-log2n", "14")
     d = json.loads(lines[0])
-    assert d["scaling"] == "strong" and d["config"]["workload"].startswith("c4")
+    assert d["scaling"] == "weak" and d["config"]["workload"].startswith("c2")
     assert _run({"WORLD_SIZE": "2", "RANK": "1"}, "--gpus", "2", "--steps", "1", "--warmup", "1") == []
