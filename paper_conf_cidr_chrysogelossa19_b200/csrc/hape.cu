@@ -25,6 +25,7 @@
 
 #include "hape.h"
 #include "kernels.cuh"
+#include "join_oa.cuh"
 #include "nonpart.cuh"
 
 using namespace hape;
@@ -198,7 +199,9 @@ static hape_status make_plan(const hape_join* h, uint64_t n_r, uint64_t n_s, hap
     b1 = (uint32_t)c.radix_bits[0];
     b2 = passes == 2 ? (uint32_t)std::max(0, c.radix_bits[1]) : 0u;
   } else if (passes == 1) {
-    b1 = std::min(need, kMaxBitsPerPass);
+    // at least 2 co-partitions: k_join_oa's free-slot test needs a
+    // co-partition other than q to exist (join_oa.cuh)
+    b1 = std::max(1u, std::min(need, kMaxBitsPerPass));
     b2 = 0;
   } else {
     b1 = std::min((need + 1) / 2, kMaxBitsPerPass);
@@ -288,6 +291,17 @@ static bool use_joint(const hape_plan& pl) {
   static const int env = [] { const char* e = getenv("HAPE_JOINT"); return e ? atoi(e) : 1; }();
   return env != 0 && pl.passes == 2 && pl.bits[0] + pl.bits[1] <= 16 && pl.bits[0] + pl.bits[1] >= 6 &&
          pl.bits[1] >= 1;
+}
+
+// Plans the joint histogram cannot count (one pass, or B1 + B2 > 16) still
+// claim their scatter runs: each pass counts only its bucket totals (k_hist
+// without per-CTA rows), a one-CTA-per-row scan turns the totals into bounds
+// and claim cursors, and the scatter claims runs from the cursors (the
+// per-CTA offset form costs 0.38-0.49 of the HBM roofline at 2^20 buckets:
+// runs of a few tuples per CTA chunk).  HAPE_CLAIM=0 keeps the per-CTA form.
+static bool use_claim(const hape_plan& pl) {
+  static const int env = [] { const char* e = getenv("HAPE_CLAIM"); return e ? atoi(e) : 1; }();
+  return env != 0 && !use_joint(pl);
 }
 
 static uint32_t joint_grid(const hape_join* h, uint32_t nchunks) {
@@ -508,8 +522,74 @@ static hape_status launch_join_m(hape_join* h, const JoinArgs& a, bool mat, uint
 #undef HAPE_JN_SU
 }
 
+// Open-addressing build+probe (join_oa.cuh).  Shape: 256 threads for
+// 8-byte R tuples, 512 for 16-byte ones (the R chunk lives in registers:
+// OA_CAPMAX / NC tuples per thread); NTAB = 2 tables (one barrier per stage)
+// when two still fit 2+ CTAs per SM, else 1; U = 2 S tuples per thread per
+// batch.  HAPE_OA_NTAB / HAPE_OA_U / HAPE_OA_SB (extra slot bits) tune the
+// int32 form; HAPE_JN_OA=0 selects the chained-table kernel (k_build_probe).
+template <int KW, int PRW, int PSW, bool MAT, bool IDENT, int NC, int NTAB, int U>
+static hape_status launch_oa_t(hape_join* h, const JoinArgs& a_in, uint32_t* ctas_out) {
+  auto kern = k_join_oa<KW, PRW, PSW, MAT, IDENT, NC, NTAB, U>;
+  JoinArgs a = a_in;
+  constexpr uint32_t capmax = (uint32_t)((OA_CAPMAX + NC - 1) / NC) * NC;
+  a.cap = std::min(a.cap, capmax);
+  static const int sb_extra = env_int("HAPE_OA_SB", 0);
+  const int sb = std::max(6, std::min(15, (int)ceil_log2_u64((uint64_t)a.cap + 1) + sb_extra));
+  a.slot_bits = (uint32_t)sb;
+  const size_t smem = oa_smem_bytes<KW, PRW, NC, NTAB>((uint32_t)sb);
+  if (smem > 200 * 1024) return fail(h, HAPE_ERR_UNSUPPORTED, "open-addressing table does not fit: %zu B", smem);
+  static uint64_t attr_dev = 0;
+  CKS(smem_attr(h, kern, 200 * 1024, attr_dev));
+  int per_sm = 0;
+  CK(h, cudaOccupancyMaxActiveBlocksPerMultiprocessor(&per_sm, kern, NC, smem));
+  if (per_sm < 1) return fail(h, HAPE_ERR_UNSUPPORTED, "open-addressing build+probe does not fit");
+  const unsigned grid = (unsigned)(per_sm * h->num_sms);
+  *ctas_out = grid;
+  kern<<<grid, NC, smem, h->stream>>>(a);
+  CK_LAUNCH(h);
+  return HAPE_OK;
+}
+
+template <int KW, int PRW, int PSW, bool MAT, bool IDENT>
+static hape_status launch_oa_m(hape_join* h, const JoinArgs& a, uint32_t* ctas) {
+  constexpr bool W8 = sizeof(Tup<KW, PRW>) == 8;
+  constexpr int NC = W8 ? 256 : 512;
+  if constexpr (KW == 4 && PRW == 4 && PSW == 4 && !MAT && !IDENT) {
+    static const int ntab = env_int("HAPE_OA_NTAB", 2), u = env_int("HAPE_OA_U", 2);
+    if (ntab == 1) {
+      if (u == 1) return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, 1, 1>(h, a, ctas);
+      if (u == 4) return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, 1, 4>(h, a, ctas);
+      return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, 1, 2>(h, a, ctas);
+    }
+    if (u == 1) return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, 2, 1>(h, a, ctas);
+    if (u == 4) return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, 2, 4>(h, a, ctas);
+    return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, 2, 2>(h, a, ctas);
+  } else {
+    return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, W8 ? 2 : 1, 2>(h, a, ctas);
+  }
+}
+
+template <int KW, int PRW, int PSW>
+static hape_status launch_oa_w(hape_join* h, const JoinArgs& a, bool mat, uint32_t* ctas) {
+  const bool ident = h->cfg.part_fn == HAPE_PART_IDENTITY;
+  if (mat) return ident ? launch_oa_m<KW, PRW, PSW, true, true>(h, a, ctas)
+                        : launch_oa_m<KW, PRW, PSW, true, false>(h, a, ctas);
+  return ident ? launch_oa_m<KW, PRW, PSW, false, true>(h, a, ctas)
+               : launch_oa_m<KW, PRW, PSW, false, false>(h, a, ctas);
+}
+
 static hape_status launch_join(hape_join* h, int kw, int prw, int psw, const JoinArgs& a, bool mat,
                                uint32_t* ctas) {
+  static const int oa = env_int("HAPE_JN_OA", 1);
+  if (oa) {
+    if (kw == 4) {
+      if (prw == 4) return psw == 4 ? launch_oa_w<4, 4, 4>(h, a, mat, ctas) : launch_oa_w<4, 4, 8>(h, a, mat, ctas);
+      return psw == 4 ? launch_oa_w<4, 8, 4>(h, a, mat, ctas) : launch_oa_w<4, 8, 8>(h, a, mat, ctas);
+    }
+    if (prw == 4) return psw == 4 ? launch_oa_w<8, 4, 4>(h, a, mat, ctas) : launch_oa_w<8, 4, 8>(h, a, mat, ctas);
+    return psw == 4 ? launch_oa_w<8, 8, 4>(h, a, mat, ctas) : launch_oa_w<8, 8, 8>(h, a, mat, ctas);
+  }
   if (kw == 4) {
     if (prw == 4) return psw == 4 ? launch_join_m<4, 4, 4>(h, a, mat, ctas) : launch_join_m<4, 4, 8>(h, a, mat, ctas);
     return psw == 4 ? launch_join_m<4, 8, 4>(h, a, mat, ctas) : launch_join_m<4, 8, 8>(h, a, mat, ctas);
@@ -577,7 +657,7 @@ static CallLayout layout_for(const hape_join* h, const hape_plan& pl, uint64_t n
   for (int s = 0; s < 2; s++) {
     SideLayout& S = L.side[s];
     S.cps1 = cps_for(h, ns[s], 1);
-    S.hist1 = cv.take(P1 * (use_joint(pl) ? 1 : S.cps1) * 4);  // joint path: pass-1 claim cursors
+    S.hist1 = cv.take(P1 * (use_joint(pl) || use_claim(pl) ? 1 : S.cps1) * 4);  // joint / claim: pass-1 cursors
     S.bounds1 = cv.take((P1 + 1) * 4);
     if (pl.passes == 2 && use_joint(pl)) {
       S.cps2 = cps_for(h, ns[s], (uint32_t)P1);
@@ -587,7 +667,7 @@ static CallLayout layout_for(const hape_join* h, const hape_plan& pl, uint64_t n
       S.part = cv.take((size_t)S.nparts * Q * 2);
     } else if (pl.passes == 2) {
       S.cps2 = cps_for(h, ns[s], (uint32_t)P1);
-      S.hist2 = cv.take(Q * S.cps2 * 4);
+      S.hist2 = cv.take(Q * (use_claim(pl) ? 1 : S.cps2) * 4);
       S.bounds2 = cv.take((Q + 1) * 4);
     }
   }
@@ -635,6 +715,15 @@ static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const
   // hold the pass-1 / pass-2 cursors, rowsum1 the row totals, rowsum2 the
   // spilled counts (both zeroed per call).
   const bool joint = use_joint(pl);
+  const bool claim = use_claim(pl);
+  // claim form: totals -> cursors (the scan reads them as a one-CTA histogram)
+  auto totals_scan = [&](SegMap m, uint32_t P, size_t cur_off, size_t rs_off, size_t bnd_off) {
+    const size_t rows = (size_t)m.nseg * P;
+    CK(h, cudaMemcpyAsync(at<uint32_t>(h, cur_off), at<uint32_t>(h, rs_off), rows * 4, cudaMemcpyDeviceToDevice,
+                          h->stream));
+    return launch_scan(h, SegMap{m.bounds, m.nseg, 1u, m.n}, P, at<uint32_t>(h, cur_off), at<uint32_t>(h, rs_off),
+                       at<uint32_t>(h, bnd_off));
+  };
   auto hist1 = [&](int s) {
     // the persistent joint-histogram CTAs take one contiguous range each (the
     // claiming scatters do not depend on the histogram's chunking)
@@ -642,7 +731,8 @@ static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const
       return launch_hist_joint(h, kw, io[s].in, SegMap{nullptr, 1u, L.side[s].nparts, io[s].in.n}, bf1, bf2, P1, P2,
                                at<uint32_t>(h, L.side[s].rowsum1),
                                at<uint16_t>(h, L.side[s].part), at<uint32_t>(h, L.side[s].rowsum2));
-    return launch_hist(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1));
+    return launch_hist(h, kw, io[s].in, m1[s], bf1, P1, claim ? nullptr : at<uint32_t>(h, L.side[s].hist1),
+                       at<uint32_t>(h, L.side[s].rowsum1));
   };
   auto scan1 = [&](int s) {
     if (joint)
@@ -650,23 +740,28 @@ static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const
                                  at<uint32_t>(h, L.side[s].rowsum2), at<uint32_t>(h, L.side[s].rowsum1), P1, P2,
                                  at<uint32_t>(h, L.side[s].bounds1), at<uint32_t>(h, L.side[s].hist1),
                                  at<uint32_t>(h, L.side[s].bounds2), at<uint32_t>(h, L.side[s].hist2));
+    if (claim) return totals_scan(m1[s], P1, L.side[s].hist1, L.side[s].rowsum1, L.side[s].bounds1);
     return launch_scan(h, m1[s], P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1),
                        at<uint32_t>(h, L.side[s].bounds1));
   };
   auto scatter1 = [&](int s) {
-    return launch_scatter(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), io[s].p1, joint);
+    return launch_scatter(h, kw, io[s].in, m1[s], bf1, P1, at<uint32_t>(h, L.side[s].hist1), io[s].p1,
+                          joint || claim);
   };
   auto hist2 = [&](int s) {
     if (joint) return HAPE_OK;
-    return launch_hist(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), at<uint32_t>(h, L.side[s].rowsum2));
+    return launch_hist(h, kw, s2[s], m2[s], bf2, P2, claim ? nullptr : at<uint32_t>(h, L.side[s].hist2),
+                       at<uint32_t>(h, L.side[s].rowsum2));
   };
   auto scan2 = [&](int s) {
     if (joint) return HAPE_OK;
+    if (claim) return totals_scan(m2[s], P2, L.side[s].hist2, L.side[s].rowsum2, L.side[s].bounds2);
     return launch_scan(h, m2[s], P2, at<uint32_t>(h, L.side[s].hist2), at<uint32_t>(h, L.side[s].rowsum2),
                        at<uint32_t>(h, L.side[s].bounds2));
   };
   auto scatter2 = [&](int s) {
-    return launch_scatter(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), io[s].p2, joint);
+    return launch_scatter(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), io[s].p2,
+                          joint || claim);
   };
   if (side1_ready) {
     for (int s = 0; s < nside; s++) {
@@ -888,6 +983,7 @@ static hape_status local_join(hape_join* h, const Src loc_in[2], const MatOut& m
     ja.bR = fb[0]; ja.bS = fb[1];
     ja.items = at<uint2>(h, L.items); ja.n_items = ctrs;
     ja.cap = pl.build_cap; ja.slice = pl.probe_slice; ja.slot_bits = pl.slot_bits;
+    ja.qmask = Q - 1;
     ja.acc = at<unsigned long long>(h, L.acc);
     ja.out_r = mo.r; ja.out_s = mo.s; ja.out_cap = mo.on ? mo.cap : 0;
     ja.out_ctr = at<unsigned long long>(h, L.out_ctr);

@@ -347,7 +347,7 @@ k_hist(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ hist
   const uint32_t row0 = seg * P;
   for (uint32_t p = threadIdx.x; p < P; p += HIST_THREADS) {
     uint32_t c = sh_cnt[p];
-    hist[(size_t)(row0 + p) * m.cps + j] = c;
+    if (hist) hist[(size_t)(row0 + p) * m.cps + j] = c;  // (claiming passes need the totals only)
     if (c) atomicAdd(&rowsum[row0 + p], c);
   }
 }
@@ -952,6 +952,7 @@ struct JoinArgs {
   uint32_t pf_bytes;                         // L2 prefetch window at the head of each S slice (0 = off)
   uint32_t nrb;                              // R-chunk ring buffers (1 or 2)
   uint32_t nsb;                              // SR kernels: staged S tiles in the ring (>= 2)
+  uint32_t qmask;                            // co-partitions - 1: q = h(key) & qmask (k_join_oa)
 };
 
 struct JnStage {

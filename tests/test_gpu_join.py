@@ -128,7 +128,8 @@ def test_c1_full_with_pairs_vs_oracle():
 
 
 @pytest.mark.parametrize("passes,bits", [(1, (0, 0)), (1, (4, 0)), (1, (11, 0)), (2, (3, 5)),
-                                         (2, (8, 8)), (2, (12, 2)), (2, (6, 12))])
+                                         (2, (8, 8)), (2, (12, 2)), (2, (6, 12)), (2, (10, 10)),
+                                         (2, (12, 12)), (1, (12, 0))])
 def test_metamorphic_plans_identical(passes, bits):
     wl = datagen.make("c2", n_r=1 << 20, n_s=(1 << 20) + 3)
     ref = provenance.expected_from_workload(wl)
@@ -381,6 +382,57 @@ def test_joint_histogram_skewed_join_vs_oracle():
     want = oracle_res(rk, rp, sk, sp)
     res = joiner(torch.int32, radix_passes=2, radix_bits=(8, 8)).join(cuda(rk), cuda(rp), cuda(sk), cuda(sp))
     check(res, want)
+
+
+@pytest.mark.parametrize("identity", [False, True])
+def test_open_addressing_refill_cases(identity):
+    """k_join_oa's free-slot test is "the slot's key is in another
+    co-partition".  Key 0 is the initial fill key (h(0) = 0: co-partition 0)
+    and consecutive stages of ONE co-partition (R chunks of an oversized R
+    side, and > grid S slices of a hot S side on one CTA) must refill."""
+    rng = np.random.default_rng(99)
+    hot = 1 << 23
+    rk = np.concatenate([np.zeros(3, np.int32), np.full(7000, 1, np.int32), rng.integers(2, 50, 40000).astype(np.int32)])
+    sk = np.concatenate([np.zeros(hot, np.int32), np.full(1000, 1, np.int32), rng.integers(0, 60, 5000).astype(np.int32)])
+    rp = rng.integers(-2**31, 2**31, len(rk)).astype(np.int32)
+    sp = rng.integers(-2**31, 2**31, len(sk)).astype(np.int32)
+    want = oracle_res(rk, rp, sk, sp)
+    res = joiner(torch.int32, identity=identity).join(cuda(rk), cuda(rp), cuda(sk), cuda(sp))
+    check(res, want)
+    assert res.n_items > 444
+
+
+@pytest.mark.parametrize("env", [dict(HAPE_JOINT="0"), dict(HAPE_JOINT="0", HAPE_CLAIM="0"),
+                                 dict(HAPE_JN_OA="0"), dict(HAPE_OA_NTAB="1"), dict(HAPE_OA_U="4"),
+                                 dict(HAPE_OA_U="1")])
+def test_alternative_kernel_forms_vs_oracle(env):
+    # the retained alternatives, each read once per process (child process):
+    # HAPE_JOINT=0 the per-pass totals + claiming scatters (the path of plans
+    # with bits[0]+bits[1] > 16), HAPE_CLAIM=0 per-CTA offset scatters,
+    # HAPE_JN_OA=0 the chained-table build+probe, HAPE_OA_* table shapes
+    import subprocess
+    import sys
+    import os
+    code = r'''
+import numpy as np, torch, datagen, oracle
+from paper_conf_cidr_chrysogelossa19_b200 import RadixJoin
+for cfg, nr, ns, kdt, bits, uq in (("c2", 1 << 20, (1 << 20) + 333, torch.int32, (8, 8), False),
+                                   ("c2", 1 << 20, (1 << 20) + 333, torch.int32, (8, 8), True),
+                                   ("c3", 1 << 18, 1 << 20, torch.int64, (8, 8), False),
+                                   ("dup", 9000, 12000, torch.int32, (9, 9), False)):
+    wl = datagen.make(cfg, n_r=nr, n_s=ns, **(dict(dup_domain=300) if cfg == "dup" else {}))
+    want = oracle.join(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload)
+    d = lambda a: torch.from_numpy(np.ascontiguousarray(a)).cuda()
+    with RadixJoin(key_dtype=kdt, radix_passes=2, radix_bits=bits, r_unique=uq) as j:
+        r = j.join(d(wl.R.key), d(wl.R.payload), d(wl.S.key), d(wl.S.payload))
+    got = dict(count=r.match_count, sum_r=r.sum_r_payload, sum_s=r.sum_s_payload, checksum=r.pair_checksum)
+    assert got == {k: want[k] for k in got}, (cfg, got, want)
+print("ok")
+'''
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    e = dict(os.environ, PYTHONPATH=root, **env)
+    r = subprocess.run([sys.executable, "-c", code], cwd=root, env=e, capture_output=True, text=True, timeout=600)
+    assert r.returncode == 0 and "ok" in r.stdout, r.stdout + r.stderr
 
 
 def test_separate_pass2_histogram_path_vs_oracle():
