@@ -43,6 +43,12 @@ constexpr int OA_CAPMAX = 3072;  // R tuples per stage (registers: OA_CAPMAX / N
 #ifndef OA_MINB
 #define OA_MINB 3
 #endif
+// 8-byte tuples: one 64-bit CAS of the whole tuple (OA_CAS64 = 1) or a 32-bit
+// CAS of the key then the payload store (0; 64-bit shared CAS measured ~6x
+// slower per build on B200)
+#ifndef OA_CAS64
+#define OA_CAS64 0
+#endif
 
 // a key that is NOT in co-partition q (fill value of a refilled table):
 // h(0) = 0 for all three partition functions, and h(1) is odd for each
@@ -68,7 +74,7 @@ __device__ __forceinline__ void oa_insert(Tup<KW, PRW>* T, uint32_t smask, uint3
                                           uint32_t q, uint32_t qmask) {
   using K = typename UW<KW>::T;
   uint32_t s = jn_slot<KW>(x.k, sb);
-  if constexpr (sizeof(Tup<KW, PRW>) == 8) {
+  if constexpr (sizeof(Tup<KW, PRW>) == 8 && OA_CAS64) {
     // (the only 8-byte tuple is (u32 key, u32 payload): key = low word)
     static_assert(KW == 4 && PRW == 4, "8-byte tuple layout");
     unsigned long long* T64 = reinterpret_cast<unsigned long long*>(T);

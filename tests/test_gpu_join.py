@@ -400,16 +400,31 @@ def test_open_addressing_refill_cases(identity):
     res = joiner(torch.int32, identity=identity).join(cuda(rk), cuda(rp), cuda(sk), cuda(sp))
     check(res, want)
     assert res.n_items > 444
+    # the same through the open-addressing form (child process: env read once)
+    import subprocess, sys, os
+    root = os.path.dirname(os.path.dirname(os.path.abspath(__file__)))
+    np.savez("/tmp/_oa_refill.npz", rk=rk, rp=rp, sk=sk, sp=sp)
+    code = (
+        "import numpy as np, torch\n"
+        "from paper_conf_cidr_chrysogelossa19_b200 import RadixJoin\n"
+        "z = np.load('/tmp/_oa_refill.npz'); d = lambda a: torch.from_numpy(z[a]).cuda()\n"
+        f"j = RadixJoin(key_dtype=torch.int32, identity={identity})\n"
+        "r = j.join(d('rk'), d('rp'), d('sk'), d('sp'))\n"
+        "print(r.match_count, r.sum_r_payload, r.sum_s_payload, r.pair_checksum)\n")
+    r = subprocess.run([sys.executable, "-c", code], cwd=root, capture_output=True, text=True, timeout=600,
+                       env=dict(os.environ, HAPE_JN_OA="1", PYTHONPATH=root))
+    assert r.returncode == 0, r.stderr
+    assert r.stdout.split() == [str(want[k]) for k in ("count", "sum_r", "sum_s", "checksum")]
 
 
 @pytest.mark.parametrize("env", [dict(HAPE_JOINT="0"), dict(HAPE_JOINT="0", HAPE_CLAIM="0"),
-                                 dict(HAPE_JN_OA="0"), dict(HAPE_OA_NTAB="1"), dict(HAPE_OA_U="4"),
-                                 dict(HAPE_OA_U="1")])
+                                 dict(HAPE_JN_OA="1"), dict(HAPE_JN_OA="1", HAPE_OA_NTAB="1"),
+                                 dict(HAPE_JN_OA="1", HAPE_OA_U="4"), dict(HAPE_JN_OA="1", HAPE_OA_U="1")])
 def test_alternative_kernel_forms_vs_oracle(env):
     # the retained alternatives, each read once per process (child process):
     # HAPE_JOINT=0 the per-pass totals + claiming scatters (the path of plans
     # with bits[0]+bits[1] > 16), HAPE_CLAIM=0 per-CTA offset scatters,
-    # HAPE_JN_OA=0 the chained-table build+probe, HAPE_OA_* table shapes
+    # HAPE_JN_OA=1 the open-addressing build+probe, HAPE_OA_* its table shapes
     import subprocess
     import sys
     import os
