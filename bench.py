@@ -434,8 +434,11 @@ def main():
     kw, pw = rk.element_size(), rp.element_size()
     t = kw + pw
     extra = {}
+    fused = res.exchange_path == 2
     if world > 1 or args.exchange:
-        extra["devpart"] = (kw + 2 * t) * (nr_loc + ns_loc)
+        # NCCL form: destination hist + scatter into a send buffer; fused form:
+        # the destination totals only (the scatter is the exchange stage)
+        extra["devpart"] = (kw if fused else kw + 2 * t) * (nr_loc + ns_loc)
     roofline = roofline_of(res, stage_avg, ms, kw, pw, pw, materialize, peak, extra)
     roofline["peak_source"] = peak_src
     traffic = None
@@ -447,9 +450,16 @@ def main():
     roofline["traffic"] = traffic
     if stage_avg.get("exchange", 0) > 0:
         xb = t * (nr_loc + ns_loc)  # every local tuple leaves through the exchange (incl. the self segment)
-        roofline["stages"]["exchange"] = {"ms": round(stage_avg["exchange"], 4), "bytes_sent": xb,
-                                          "GB/s": round(xb / (stage_avg["exchange"] / 1000.0) / 1e9, 1),
-                                          "bound": "nvlink (NCCL all-to-allv)"}
+        xs = stage_avg["exchange"] / 1000.0
+        remote = xb * (world - 1) // max(world, 1)
+        roofline["stages"]["exchange"] = {
+            "ms": round(stage_avg["exchange"], 4), "bytes_sent": xb, "GB/s": round(xb / xs / 1e9, 1),
+            "remote_bytes": remote, "remote_GB/s": round(remote / xs / 1e9, 1),
+            "nvlink_frac": round(remote / xs / 1e9 / 900.0, 3) if world > 1 else None,
+            "form": "fused peer scatter (destination partition writes into the peers' receive buffers)"
+            if fused else "NCCL send/recv of a device-partitioned send buffer",
+            "bound": "nvlink 900 GB/s/dir per GPU (remote part); HBM 2t B/tuple (read + write)"}
+        roofline["exchange_path"] = res.exchange_path
 
     # ---- end to end through the same C ABI call with pinned host buffers
     e2e = None

@@ -57,6 +57,7 @@ class JoinResult:
     n_items: int
     kernel_launches: int
     stage_ms: dict
+    exchange_path: int = 0
 
     def as_tuple(self):
         return (self.match_count, self.sum_r_payload, self.sum_s_payload, self.pair_checksum)
@@ -99,7 +100,8 @@ def _result(st, res) -> "JoinResult":
         s_local=res.s_local, passes=res.passes, bits=(res.bits[0], res.bits[1]),
         n_partitions=res.n_partitions, n_items=res.n_items,
         kernel_launches=res.kernel_launches,
-        stage_ms={name: float(res.stage_ms[i]) for i, name in enumerate(STAGES)})
+        stage_ms={name: float(res.stage_ms[i]) for i, name in enumerate(STAGES)},
+        exchange_path=res.exchange_path)
 
 
 class RadixJoin:
@@ -239,9 +241,12 @@ class RadixJoin:
             raise HapeError(st, hape_last_error(self._h))
         return _result(st, res)
 
-    def loopback_join(self, r_shards, s_shards, out_r=None, out_s=None, raise_on_capacity: bool = True):
+    def loopback_join(self, r_shards, s_shards, out_r=None, out_s=None, raise_on_capacity: bool = True,
+                      peer: bool = False):
         """hape_debug_loopback_join: len(r_shards) simulated ranks on this GPU
-        (every device step of the G>1 path; device copies stand in for NCCL).
+        (every device step of the G>1 path; device copies stand in for NCCL,
+        or, with peer=True, the fused peer-scatter exchange into one receive
+        buffer per simulated rank).
         r_shards / s_shards: lists of (key, payload) CUDA tensor pairs.
         Returns (total JoinResult, [per-destination JoinResult])."""
         G = len(r_shards)
@@ -252,7 +257,8 @@ class RadixJoin:
         self._order_inputs()
         per = (hape_join_result * G)()
         tot = hape_join_result()
-        st = hape_debug_loopback_join(self._h, G, [r for r, _ in rels], [s for _, s in rels], out, per, tot)
+        st = hape_debug_loopback_join(self._h, G, int(peer), [r for r, _ in rels], [s for _, s in rels], out, per,
+                                      tot)
         if st != HAPE_OK and not (st == HAPE_ERR_OUTPUT_CAPACITY and not raise_on_capacity):
             raise HapeError(st, hape_last_error(self._h))
         return _result(st, tot), [_result(st, per[d]) for d in range(G)]

@@ -36,7 +36,8 @@ EXPORTED = ["hape_version", "hape_status_string", "hape_join_create", "hape_radi
             "hape_join_destroy", "hape_last_error", "hape_join_plan", "hape_debug_partition",
             "hape_nccl_unique_id", "hape_nccl_comm_init", "hape_nccl_comm_destroy",
             "hape_exchange_plan", "hape_nonpartitioned_join", "hape_coprocess_join",
-            "hape_host_partition", "hape_join_stream", "hape_debug_route", "hape_debug_loopback_join"]
+            "hape_host_partition", "hape_join_stream", "hape_debug_route", "hape_debug_loopback_join",
+            "hape_peer_plan"]
 
 
 class hape_join_config(ctypes.Structure):
@@ -67,7 +68,8 @@ class hape_join_result(ctypes.Structure):
                 ("r_local", ctypes.c_uint64), ("s_local", ctypes.c_uint64),
                 ("passes", ctypes.c_uint32), ("bits", ctypes.c_uint32 * 2),
                 ("n_partitions", ctypes.c_uint32), ("n_items", ctypes.c_uint32),
-                ("kernel_launches", ctypes.c_uint32), ("stage_ms", ctypes.c_float * HAPE_NSTAGES)]
+                ("kernel_launches", ctypes.c_uint32), ("stage_ms", ctypes.c_float * HAPE_NSTAGES),
+                ("exchange_path", ctypes.c_uint32)]
 
 
 class hape_coprocess_config(ctypes.Structure):
@@ -126,12 +128,15 @@ def _load() -> ctypes.CDLL:
     lib.hape_exchange_plan.restype = ctypes.c_int
     lib.hape_exchange_plan.argtypes = [ctypes.c_int, ctypes.c_int, P(ctypes.c_uint64),
                                        P(ctypes.c_uint64), P(ctypes.c_uint64), P(ctypes.c_uint64)]
+    lib.hape_peer_plan.restype = ctypes.c_int
+    lib.hape_peer_plan.argtypes = [ctypes.c_int, ctypes.c_int, P(ctypes.c_uint64), P(ctypes.c_uint64),
+                                   P(ctypes.c_uint64), P(ctypes.c_uint64)]
     lib.hape_join_stream.restype = ctypes.c_int
     lib.hape_join_stream.argtypes = [vp, P(vp)]
     lib.hape_debug_route.restype = ctypes.c_int
     lib.hape_debug_route.argtypes = [vp, P(hape_relation), ctypes.c_int, ctypes.c_int, vp, vp, vp]
     lib.hape_debug_loopback_join.restype = ctypes.c_int
-    lib.hape_debug_loopback_join.argtypes = [vp, ctypes.c_int, P(hape_relation), P(hape_relation),
+    lib.hape_debug_loopback_join.argtypes = [vp, ctypes.c_int, ctypes.c_int, P(hape_relation), P(hape_relation),
                                              P(hape_output), P(hape_join_result), P(hape_join_result)]
     return lib
 
@@ -240,8 +245,19 @@ def hape_debug_route(h, rel: hape_relation, is_s: int, fanout: int, out_keys: in
     return lib.hape_debug_route(h, ctypes.byref(rel), is_s, fanout, out_keys, out_payloads, out_bounds)
 
 
-def hape_debug_loopback_join(h, world: int, R_shards, S_shards, out, per_dest, total: hape_join_result) -> int:
+def hape_debug_loopback_join(h, world: int, peer: int, R_shards, S_shards, out, per_dest,
+                             total: hape_join_result) -> int:
     Ra = (hape_relation * world)(*R_shards)
     Sa = (hape_relation * world)(*S_shards)
-    return lib.hape_debug_loopback_join(h, world, Ra, Sa, ctypes.byref(out) if out is not None else None,
+    return lib.hape_debug_loopback_join(h, world, peer, Ra, Sa, ctypes.byref(out) if out is not None else None,
                                         per_dest, ctypes.byref(total))
+
+
+def hape_peer_plan(world: int, rank: int, counts):
+    G = world
+    c = (ctypes.c_uint64 * (G * G))(*[int(x) for x in counts])
+    wo = (ctypes.c_uint64 * G)()
+    rt = ctypes.c_uint64()
+    cap = ctypes.c_uint64()
+    st = lib.hape_peer_plan(G, rank, c, wo, ctypes.byref(rt), ctypes.byref(cap))
+    return st, list(wo), int(rt.value), int(cap.value)

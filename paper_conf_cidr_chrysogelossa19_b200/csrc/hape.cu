@@ -90,6 +90,19 @@ struct hape_join {
   DevBuf cpst[2][4];
   cudaEvent_t ev_h2d[2][2] = {};
   bool in_coprocess = false;            // join_impl: no CUDA-graph capture (sizes change per call)
+  // G>1 peer exchange (exchange_p2p): receive buffers (IPC-exportable,
+  // grown collectively), the peers' mapped receive buffers, the device
+  // table of destination pointers per relation, pinned host scratch
+  DevBuf prx[2];
+  void* peer_rx[2][64] = {};            // opened IPC mappings (nullptr for self)
+  DevBuf peer_tab;                      // [2][G] Tup* destinations
+  DevBuf xipc;                          // IPC handle all-gather staging
+  uint32_t* h_x = nullptr;              // pinned: [2][G] cursors
+  bool p2p_failed = false;              // IPC unavailable: NCCL send/recv from then on
+  // hape_debug_loopback_join (peer form): one receive buffer per simulated rank
+  DevBuf lb_rx[2][64];
+  uint32_t xchg_path = 0;               // last call: 0 none, 1 NCCL send/recv, 2 peer scatter
+  bool peer_tab_dirty = false;          // peer_tab holds the loopback's table
 };
 
 // ---------------------------------------------------------------------------
@@ -439,6 +452,39 @@ static hape_status launch_scatter(hape_join* h, int kw, const Src& s, SegMap m, 
   return scatter_v<8, 8, AOS>(h, s, m, bf, P, offs, out, claim);
   if (s.aos) { HAPE_SC_DISPATCH(true) } else { HAPE_SC_DISPATCH(false) }
 #undef HAPE_SC_DISPATCH
+}
+
+// the fused destination partition + exchange scatter (k_scatter PEER): SoA
+// caller columns in, claimed runs straight into each destination's buffer
+template <int KW, int PW, bool IDENT>
+static hape_status peer_scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* offs,
+                                  void* const* peers) {
+  using C = ScCfg<512, 13, 2, 2>;
+  using Cw = typename std::conditional<KW + PW <= 8, C, ScCfg<384, 9, 2, 2>>::type;
+  auto kern = k_scatter<KW, PW, false, Cw, IDENT, true, true>;
+  const size_t smem = ScLayout<KW, PW, false, Cw>::bytes(P, true);
+  static uint64_t attr_dev = 0;
+  CKS(smem_attr(h, kern, 220 * 1024, attr_dev));
+  const unsigned grid = m.nseg * m.cps;
+  if (grid == 0) return HAPE_OK;
+  kern<<<grid, Cw::NT, smem, h->stream>>>(s.in, m, bf, P, offs, nullptr,
+                                         reinterpret_cast<Tup<KW, PW>* const*>(peers));
+  CK_LAUNCH(h);
+  return HAPE_OK;
+}
+
+static hape_status launch_peer_scatter(hape_join* h, int kw, const Src& s, SegMap m, BitField bf, uint32_t P,
+                                       uint32_t* offs, void* const* peers) {
+  if (s.aos) return fail(h, HAPE_ERR_UNSUPPORTED, "peer scatter reads SoA columns");
+  const int pw = s.pw;
+  const bool id = h->cfg.part_fn == HAPE_PART_IDENTITY;
+#define HAPE_PS(KW, PW) return id ? peer_scatter_t<KW, PW, true>(h, s, m, bf, P, offs, peers) \
+                                 : peer_scatter_t<KW, PW, false>(h, s, m, bf, P, offs, peers)
+  if (kw == 4 && pw == 4) HAPE_PS(4, 4);
+  if (kw == 4) HAPE_PS(4, 8);
+  if (pw == 4) HAPE_PS(8, 4);
+  HAPE_PS(8, 8);
+#undef HAPE_PS
 }
 
 // Build+probe shape: SR kernels (SU > 0) stage S through a smem tile ring of
@@ -915,6 +961,173 @@ static hape_status exchange(hape_join* h, Src in[2], Src out[2]) {
     CKN(h, ncclGroupEnd());
     out[s] = Src{PartIn{nullptr, nullptr, h->recv[s].p}, true, (uint32_t)rtot, in[s].pw};
   }
+  h->xchg_path = 1;
+  return HAPE_OK;
+}
+
+// ---------------------------------------------------------------------------
+// G>1, fused form: the destination partition's scatter
+// writes its claimed runs straight into the destination ranks' receive
+// buffers over NVLink (peer pointers from CUDA IPC handles exchanged once per
+// buffer growth), so the exchange costs no send buffer, no second read and
+// no separate transfer: the NVLink traffic overlaps the partitioning tile by
+// tile.  The router + mem-move of P643-656 as ONE kernel.
+// ---------------------------------------------------------------------------
+extern "C" hape_status hape_peer_plan(int world_size, int rank, const uint64_t* counts, uint64_t* write_off,
+                                      uint64_t* recv_total, uint64_t* recv_capacity) {
+  if (world_size < 1 || rank < 0 || rank >= world_size || !counts || !write_off || !recv_total || !recv_capacity)
+    return HAPE_ERR_INVALID_ARG;
+  const int G = world_size;
+  uint64_t mx = 0;
+  for (int d = 0; d < G; d++) {
+    uint64_t t = 0, base = 0;
+    for (int src = 0; src < G; src++) {
+      const uint64_t x = counts[(size_t)src * G + d];
+      if (src < rank) base += x;
+      t += x;
+    }
+    write_off[d] = base;
+    if (d == rank) *recv_total = t;
+    mx = std::max(mx, t);
+  }
+  *recv_capacity = mx;
+  return HAPE_OK;
+}
+
+static BitField dest_field(const hape_join* h, uint32_t G) {
+  const uint32_t g = ceil_log2_u64((uint64_t)G);
+  const uint32_t HW = key_width(h->cfg) * 8;
+  return BitField{g ? HW - g : 0u, G - 1};  // destination = top g bits of h (R14)
+}
+
+// per-destination totals of one relation (totals-only histogram, += into
+// `totals`, which the caller zeroes)
+static hape_status route_totals(hape_join* h, const Src& in, uint32_t G, uint32_t* totals) {
+  const SegMap m{nullptr, 1u, cps_for(h, in.n, 1), in.n};
+  return launch_hist(h, key_width(h->cfg), in, m, dest_field(h, G), G, nullptr, totals);
+}
+
+static hape_status route_peer(hape_join* h, const Src& in, uint32_t G, uint32_t* cursors, void* const* peers) {
+  const SegMap m{nullptr, 1u, cps_for(h, in.n, 1), in.n};
+  return launch_peer_scatter(h, key_width(h->cfg), in, m, dest_field(h, G), G, cursors, peers);
+}
+
+static void close_peers(hape_join* h, int s) {
+  for (auto& p : h->peer_rx[s])
+    if (p) {
+      cudaIpcCloseMemHandle(p);
+      p = nullptr;
+    }
+}
+
+// returns HAPE_ERR_UNSUPPORTED (on every rank alike) when some rank could not
+// map its peers' buffers; the caller then runs the NCCL send/recv exchange
+static hape_status exchange_p2p(hape_join* h, Src in[2], Src out[2]) {
+  const int G = std::max(1, h->cfg.world_size), me = h->cfg.rank;
+  const int kw = key_width(h->cfg);
+  const size_t nl = (size_t)2 * G, nb = (size_t)G * nl;
+  // xb: totals [2][G] | gathered [G][2][G] | cursors [2][G] | flag / barrier words
+  CKS(ensure(h, h->xb, (nl + nb + nl + 8) * 4));
+  uint32_t* tot = static_cast<uint32_t*>(h->xb.p);
+  uint32_t* gat = tot + nl;
+  uint32_t* cur = gat + nb;
+  uint32_t* word = cur + nl;
+  CK(h, cudaMemsetAsync(tot, 0, nl * 4, h->stream));
+  mark(h, HAPE_STAGE_DEVPART);
+  for (int s = 0; s < 2; s++) CKS(route_totals(h, in[s], (uint32_t)G, tot + s * G));
+  // count exchange -- also the start barrier: a rank's all-gather runs after
+  // its previous local join (stream order), and no rank scatters into a peer
+  // before every rank has joined the all-gather
+  CKN(h, ncclAllGather(tot, gat, nl, ncclUint32, h->comm, h->stream));
+  if (h->h_bounds_cap < nb) {
+    if (h->h_bounds) cudaFreeHost(h->h_bounds);
+    h->h_bounds = nullptr;
+    h->h_bounds_cap = 0;
+    CK(h, cudaMallocHost(&h->h_bounds, nb * 4));
+    h->h_bounds_cap = nb;
+  }
+  CK(h, cudaMemcpyAsync(h->h_bounds, gat, nb * 4, cudaMemcpyDeviceToHost, h->stream));
+  CK(h, cudaStreamSynchronize(h->stream));
+  const uint32_t* c = h->h_bounds;  // c[src*nl + s*G + d]
+  size_t tb[2];
+  uint64_t rtot[2], need[2];
+  for (int s = 0; s < 2; s++) {
+    tb[s] = tup_bytes(kw, in[s].pw);
+    std::vector<uint64_t> counts((size_t)G * G), off(G);
+    for (int src = 0; src < G; src++)
+      for (int d = 0; d < G; d++) counts[(size_t)src * G + d] = c[(size_t)src * nl + s * G + d];
+    uint64_t mx = 0;
+    hape_peer_plan(G, me, counts.data(), off.data(), &rtot[s], &mx);
+    for (int d = 0; d < G; d++) h->h_x[s * G + d] = (uint32_t)off[d];
+    if (mx >= 0xFFFFFFFFull) return fail(h, HAPE_ERR_UNSUPPORTED, "a rank receives %llu tuples >= 2^32", (unsigned long long)mx);
+    need[s] = mx * tb[s] + 16;  // the same on every rank: buffers grow together
+  }
+  bool remap = !h->peer_tab.p || h->peer_tab_dirty;
+  h->peer_tab_dirty = false;
+  for (int s = 0; s < 2; s++) {
+    if (need[s] <= h->prx[s].bytes) continue;
+    close_peers(h, s);
+    CKS(ensure(h, h->prx[s], need[s] + need[s] / 8));
+    remap = true;
+  }
+  if (remap) {
+    void* tab[2][64] = {};
+    int bad = 0;
+    if (G > 1) {
+      // all-gather the receive buffers' IPC handles, map the peers'
+      cudaIpcMemHandle_t mine[2];
+      for (int s = 0; s < 2; s++) CK(h, cudaIpcGetMemHandle(&mine[s], h->prx[s].p));
+      const size_t hb = sizeof mine;
+      CKS(ensure(h, h->xipc, hb * (G + 1)));
+      std::vector<unsigned char> all(hb * G);
+      CK(h, cudaMemcpyAsync(h->xipc.p, mine, hb, cudaMemcpyHostToDevice, h->stream));
+      CKN(h, ncclAllGather(h->xipc.p, static_cast<char*>(h->xipc.p) + hb, hb, ncclUint8, h->comm, h->stream));
+      CK(h, cudaMemcpyAsync(all.data(), static_cast<char*>(h->xipc.p) + hb, hb * G, cudaMemcpyDeviceToHost, h->stream));
+      CK(h, cudaStreamSynchronize(h->stream));
+      for (int p = 0; p < G && !bad; p++) {
+        if (p == me) continue;
+        for (int s = 0; s < 2 && !bad; s++) {
+          cudaIpcMemHandle_t hd;
+          memcpy(&hd, all.data() + hb * p + sizeof(cudaIpcMemHandle_t) * s, sizeof hd);
+          if (h->peer_rx[s][p]) cudaIpcCloseMemHandle(h->peer_rx[s][p]);
+          h->peer_rx[s][p] = nullptr;
+          if (cudaIpcOpenMemHandle(&h->peer_rx[s][p], hd, cudaIpcMemLazyEnablePeerAccess) != cudaSuccess) {
+            (void)cudaGetLastError();
+            h->peer_rx[s][p] = nullptr;
+            bad = 1;
+          }
+        }
+      }
+      // every rank takes the same path: max of the failure flags
+      CK(h, cudaMemcpyAsync(word, &bad, 4, cudaMemcpyHostToDevice, h->stream));
+      CKN(h, ncclAllReduce(word, word, 1, ncclInt32, ncclMax, h->comm, h->stream));
+      CK(h, cudaMemcpyAsync(&bad, word, 4, cudaMemcpyDeviceToHost, h->stream));
+      CK(h, cudaStreamSynchronize(h->stream));
+      if (bad) {
+        for (int s = 0; s < 2; s++) close_peers(h, s);
+        h->p2p_failed = true;
+        return fail(h, HAPE_ERR_UNSUPPORTED, "peer mapping of the receive buffers failed on some rank");
+      }
+    }
+    for (int s = 0; s < 2; s++)
+      for (int d = 0; d < G; d++) tab[s][d] = d == me ? h->prx[s].p : h->peer_rx[s][d];
+    CKS(ensure(h, h->peer_tab, nl * sizeof(void*)));
+    std::vector<void*> flat(nl);
+    for (int s = 0; s < 2; s++)
+      for (int d = 0; d < G; d++) flat[s * G + d] = tab[s][d];
+    CK(h, cudaMemcpyAsync(h->peer_tab.p, flat.data(), nl * sizeof(void*), cudaMemcpyHostToDevice, h->stream));
+    CK(h, cudaStreamSynchronize(h->stream));
+  }
+  // this rank's segment start inside every destination's buffer
+  CK(h, cudaMemcpyAsync(cur, h->h_x, nl * 4, cudaMemcpyHostToDevice, h->stream));
+  mark(h, HAPE_STAGE_EXCHANGE);
+  void* const* ptab = static_cast<void* const*>(h->peer_tab.p);
+  for (int s = 0; s < 2; s++) CKS(route_peer(h, in[s], (uint32_t)G, cur + s * G, ptab + s * G));
+  // completion barrier: each rank's scatter (ending in a system-scope fence)
+  // precedes its contribution, so afterwards every receive buffer is complete
+  CKN(h, ncclAllReduce(word + 1, word + 1, 1, ncclUint32, ncclSum, h->comm, h->stream));
+  for (int s = 0; s < 2; s++) out[s] = Src{PartIn{nullptr, nullptr, h->prx[s].p}, true, (uint32_t)rtot[s], in[s].pw};
+  h->xchg_path = 2;
   return HAPE_OK;
 }
 
@@ -1108,7 +1321,18 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
     CKS(stage_in(h, S, kw, psw, h->stage[2], h->stage[3], &in[1]));
   }
   Src loc[2] = {in[0], in[1]};
-  if (world > 1 || h->comm) CKS(exchange(h, in, loc));
+  h->xchg_path = 0;
+  if (world > 1 || h->comm) {
+    // fused peer-scatter exchange unless disabled (HAPE_XCHG=nccl) or the
+    // peers' buffers could not be mapped (then NCCL send/recv, every rank)
+    static const bool nccl_only = [] { const char* e = getenv("HAPE_XCHG"); return e && !strcmp(e, "nccl"); }();
+    hape_status xs = HAPE_ERR_UNSUPPORTED;
+    if (!nccl_only && !h->p2p_failed) {
+      xs = exchange_p2p(h, in, loc);
+      if (xs != HAPE_OK && xs != HAPE_ERR_UNSUPPORTED) return xs;
+    }
+    if (xs != HAPE_OK) CKS(exchange(h, in, loc));
+  }
 
   MatOut mo;
   CKS(mat_targets(h, out, &mo));
@@ -1138,6 +1362,7 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   res->n_written = mat ? std::min<uint64_t>(r[4], out->capacity) : 0;
   res->n_items = (uint32_t)(r[5] & 0xFFFFFFFFu);
   fill_plan_fields(res, pl, loc[0].n, loc[1].n);
+  res->exchange_path = h->xchg_path;
   if (mat && out->mem == HAPE_MEM_HOST && res->n_written) {
     CK(h, cudaMemcpyAsync(out->r_payload, mo.r, res->n_written * prw, cudaMemcpyDeviceToHost, h->stream));
     CK(h, cudaMemcpyAsync(out->s_payload, mo.s, res->n_written * psw, cudaMemcpyDeviceToHost, h->stream));
@@ -1160,7 +1385,7 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
 // transport replaced by device-to-device copies of the same segments to the
 // same receive offsets.
 // ---------------------------------------------------------------------------
-static hape_status loopback_impl(hape_join* h, int G, const hape_relation* Rs, const hape_relation* Ss,
+static hape_status loopback_impl(hape_join* h, int G, bool peer, const hape_relation* Rs, const hape_relation* Ss,
                                  const hape_output* out, hape_join_result* per_dest, hape_join_result* total) {
   const hape_join_config& c = h->cfg;
   const int kw = key_width(c), prw = pay_width(c.r_payload_type), psw = pay_width(c.s_payload_type);
@@ -1184,36 +1409,79 @@ static hape_status loopback_impl(hape_join* h, int G, const hape_relation* Rs, c
   memset(total, 0, sizeof *total);
   for (int i = 0; i < HAPE_NSTAGES; i++) h->ev_used[i] = false;
   h->launches = 0;
-  // (a2-a4) route every source shard into its region of the send buffer
   size_t tb[2];
-  for (int s = 0; s < 2; s++) {
-    tb[s] = tup_bytes(kw, pws[s]);
-    CKS(ensure(h, h->send[s], ntot[s] * tb[s] + 16));
-  }
-  CKS(ensure(h, h->xb, (size_t)2 * G * (G + 1) * 4));
-  uint32_t* dbounds = static_cast<uint32_t*>(h->xb.p);
+  for (int s = 0; s < 2; s++) tb[s] = tup_bytes(kw, pws[s]);
   std::vector<uint64_t> base[2];
-  for (int s = 0; s < 2; s++) {
-    base[s].assign(G + 1, 0);
-    for (int i = 0; i < G; i++) {
-      Src in;
-      CKS(stage_in(h, &shards[s][i], kw, pws[s], h->stage[0], h->stage[1], &in));
-      CKS(route(h, in, (uint32_t)G, static_cast<char*>(h->send[s].p) + base[s][i] * tb[s],
-                dbounds + ((size_t)s * G + i) * (G + 1)));
-      base[s][i + 1] = base[s][i] + shards[s][i].n;
-    }
-  }
-  // (a5) count exchange
-  std::vector<uint32_t> hb((size_t)2 * G * (G + 1));
-  CK(h, cudaMemcpyAsync(hb.data(), dbounds, hb.size() * 4, cudaMemcpyDeviceToHost, h->stream));
-  CK(h, cudaStreamSynchronize(h->stream));
   std::vector<uint64_t> counts[2];
-  for (int s = 0; s < 2; s++) {
-    counts[s].assign((size_t)G * G, 0);
-    for (int src = 0; src < G; src++) {
-      const uint32_t* b = hb.data() + ((size_t)s * G + src) * (G + 1);
-      for (int d = 0; d < G; d++) counts[s][(size_t)src * G + d] = b[d + 1] - b[d];
+  std::vector<uint32_t> hb((size_t)2 * G * (G + 1));
+  if (!peer) {
+    // (a2-a4) route every source shard into its region of the send buffer
+    for (int s = 0; s < 2; s++) CKS(ensure(h, h->send[s], ntot[s] * tb[s] + 16));
+    CKS(ensure(h, h->xb, (size_t)2 * G * (G + 1) * 4));
+    uint32_t* dbounds = static_cast<uint32_t*>(h->xb.p);
+    for (int s = 0; s < 2; s++) {
+      base[s].assign(G + 1, 0);
+      for (int i = 0; i < G; i++) {
+        Src in;
+        CKS(stage_in(h, &shards[s][i], kw, pws[s], h->stage[0], h->stage[1], &in));
+        CKS(route(h, in, (uint32_t)G, static_cast<char*>(h->send[s].p) + base[s][i] * tb[s],
+                  dbounds + ((size_t)s * G + i) * (G + 1)));
+        base[s][i + 1] = base[s][i] + shards[s][i].n;
+      }
     }
+    // (a5) count exchange
+    CK(h, cudaMemcpyAsync(hb.data(), dbounds, hb.size() * 4, cudaMemcpyDeviceToHost, h->stream));
+    CK(h, cudaStreamSynchronize(h->stream));
+    for (int s = 0; s < 2; s++) {
+      counts[s].assign((size_t)G * G, 0);
+      for (int src = 0; src < G; src++) {
+        const uint32_t* b = hb.data() + ((size_t)s * G + src) * (G + 1);
+        for (int d = 0; d < G; d++) counts[s][(size_t)src * G + d] = b[d + 1] - b[d];
+      }
+    }
+  } else {
+    // fused form: per-destination totals of every shard (the all-gathered
+    // count matrix), then every shard's peer scatter into the destinations'
+    // receive buffers at its offset inside each
+    const size_t nt = (size_t)G * 2 * G;
+    CKS(ensure(h, h->xb, (nt + nt) * 4));
+    uint32_t* tot = static_cast<uint32_t*>(h->xb.p);  // [src][s][d]
+    uint32_t* cur = tot + nt;                           // [src][s][d] cursors
+    CK(h, cudaMemsetAsync(tot, 0, nt * 4, h->stream));
+    std::vector<Src> ins((size_t)2 * G);
+    for (int s = 0; s < 2; s++)
+      for (int i = 0; i < G; i++) {
+        CKS(stage_in(h, &shards[s][i], kw, pws[s], h->stage[0], h->stage[1], &ins[(size_t)s * G + i]));
+        CKS(route_totals(h, ins[(size_t)s * G + i], (uint32_t)G, tot + ((size_t)i * 2 + s) * G));
+      }
+    std::vector<uint32_t> ht(nt);
+    CK(h, cudaMemcpyAsync(ht.data(), tot, nt * 4, cudaMemcpyDeviceToHost, h->stream));
+    CK(h, cudaStreamSynchronize(h->stream));
+    std::vector<uint32_t> hc(nt);
+    std::vector<void*> tab((size_t)2 * G);
+    for (int s = 0; s < 2; s++) {
+      counts[s].assign((size_t)G * G, 0);
+      for (int d = 0; d < G; d++) {
+        uint64_t run = 0;
+        for (int src = 0; src < G; src++) {
+          const uint32_t x = ht[((size_t)src * 2 + s) * G + d];
+          counts[s][(size_t)src * G + d] = x;
+          hc[((size_t)src * 2 + s) * G + d] = (uint32_t)run;
+          run += x;
+        }
+        CKS(ensure(h, h->lb_rx[s][d], run * tb[s] + 16));
+        tab[(size_t)s * G + d] = h->lb_rx[s][d].p;
+      }
+    }
+    CKS(ensure(h, h->peer_tab, tab.size() * sizeof(void*)));
+    CK(h, cudaMemcpyAsync(h->peer_tab.p, tab.data(), tab.size() * sizeof(void*), cudaMemcpyHostToDevice, h->stream));
+    CK(h, cudaMemcpyAsync(cur, hc.data(), nt * 4, cudaMemcpyHostToDevice, h->stream));
+    void* const* ptab = static_cast<void* const*>(h->peer_tab.p);
+    for (int i = 0; i < G; i++)
+      for (int s = 0; s < 2; s++)
+        CKS(route_peer(h, ins[(size_t)s * G + i], (uint32_t)G, cur + ((size_t)i * 2 + s) * G, ptab + (size_t)s * G));
+    CK(h, cudaStreamSynchronize(h->stream));  // (host vectors above are the copies' sources)
+    h->peer_tab_dirty = true;                 // the exchange path re-uploads its own table
   }
   MatOut mo0;
   CKS(mat_targets(h, out, &mo0));
@@ -1225,6 +1493,10 @@ static hape_status loopback_impl(hape_join* h, int G, const hape_relation* Rs, c
       std::vector<uint64_t> soff(G), roff(G);
       uint64_t rtot = 0;
       hape_exchange_plan(G, d, counts[s].data(), soff.data(), roff.data(), &rtot);
+      if (peer) {
+        loc[s] = Src{PartIn{nullptr, nullptr, h->lb_rx[s][d].p}, true, (uint32_t)rtot, pws[s]};
+        continue;
+      }
       CKS(ensure(h, h->recv[s], rtot * tb[s] + 16));
       // the all-to-allv: source src's destination-d segment -> roff[src]
       for (int src = 0; src < G; src++) {
@@ -1481,6 +1753,7 @@ hape_status hape_join_create(const hape_join_config* cfg, hape_join** out_handle
         cudaEventCreateWithFlags(&h->ev_copy, cudaEventDisableTiming) != cudaSuccess) { st = HAPE_ERR_CUDA; break; }
     if (st != HAPE_OK) break;
     if (cudaMallocHost(&h->h_res, 16 * sizeof(unsigned long long)) != cudaSuccess) { st = HAPE_ERR_OOM; break; }
+    if (cudaMallocHost(&h->h_x, 2 * 64 * sizeof(uint32_t)) != cudaSuccess) { st = HAPE_ERR_OOM; break; }
     if (cfg->max_r || cfg->max_s) {
       hape_plan pl;
       if (make_plan(h, cfg->max_r, cfg->max_s, &pl) == HAPE_OK) {
@@ -1538,6 +1811,15 @@ hape_status hape_join_destroy(hape_join* h) {
   if (h->gexec) cudaGraphExecDestroy(h->gexec);
   if (h->small.p) cudaFree(h->small.p);
   if (h->route_ws.p) cudaFree(h->route_ws.p);
+  for (int s2 = 0; s2 < 2; s2++) {
+    close_peers(h, s2);
+    if (h->prx[s2].p) cudaFree(h->prx[s2].p);
+    for (auto& b : h->lb_rx[s2])
+      if (b.p) cudaFree(b.p);
+  }
+  if (h->peer_tab.p) cudaFree(h->peer_tab.p);
+  if (h->xipc.p) cudaFree(h->xipc.p);
+  if (h->h_x) cudaFreeHost(h->h_x);
   if (h->xb.p) cudaFree(h->xb.p);
   if (h->np_table.p) cudaFree(h->np_table.p);
   if (h->h_res) cudaFreeHost(h->h_res);
@@ -1657,12 +1939,12 @@ hape_status hape_debug_route(hape_join* h, const hape_relation* rel, int is_s, i
   }
 }
 
-hape_status hape_debug_loopback_join(hape_join* h, int world, const hape_relation* R_shards,
+hape_status hape_debug_loopback_join(hape_join* h, int world, int peer, const hape_relation* R_shards,
                                      const hape_relation* S_shards, const hape_output* out,
                                      hape_join_result* per_dest, hape_join_result* total) {
   if (!h) return HAPE_ERR_INVALID_ARG;
   try {
-    return loopback_impl(h, world, R_shards, S_shards, out, per_dest, total);
+    return loopback_impl(h, world, peer != 0, R_shards, S_shards, out, per_dest, total);
   } catch (...) {
     return fail(h, HAPE_ERR_CUDA, "unexpected C++ exception");
   }

@@ -618,9 +618,9 @@ struct ScLayout {
   static constexpr size_t RP = AOS ? 0 : (size_t)T * PW + 32;
   static constexpr size_t RAW0 = (RK + RP + 15) / 16 * 16;
   static constexpr size_t RAW = RAW0 > (size_t)T * sizeof(Tp) ? RAW0 : (size_t)T * sizeof(Tp);
-  static __host__ __device__ constexpr size_t bytes(uint32_t P) {
+  static __host__ __device__ constexpr size_t bytes(uint32_t P, bool peer = false) {
     return C::STAGES * RAW + (C::DST ? (size_t)T * 4 : 0) + (size_t)((P + 3) & ~3u) * 16 + 64 * 4 +
-           C::STAGES * 8 + 64;
+           C::STAGES * 8 + 64 + (peer ? (size_t)((P + 1) & ~1u) * 8 : 0);
   }
 };
 
@@ -652,10 +652,19 @@ __device__ __forceinline__ void sc_issue(const PartIn& in, uint32_t t0, uint32_t
 // sub-partition then land in claim order (any order is a valid partition,
 // DESIGN.md R9); the claimed regions of concurrently running tiles are
 // adjacent, so L2 still merges the partial sectors at their seams.
-template <int KW, int PW, bool AOS, class C, bool IDENT, bool CLAIM = false>
+//
+// PEER (the fused device partition + exchange of the G>1 path, SURVEY §8.f
+// NEXT-1): bucket b is destination rank b, `peer_out[b]` is that rank's
+// receive buffer (a peer pointer over NVLink, or this rank's own buffer) and
+// offsets[b] starts at this rank's segment inside it: the runs land in the
+// peers' memory straight from the staging tile -- no send buffer, no separate
+// transfer.  Every thread fences at system scope before exiting, so the
+// stores are visible to the peers once their stream-ordered barrier passes.
+template <int KW, int PW, bool AOS, class C, bool IDENT, bool CLAIM = false, bool PEER = false>
 __global__ void __launch_bounds__(C::NT, C::MINB)
 k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ offsets,
-          Tup<KW, PW>* __restrict__ out) {
+          Tup<KW, PW>* __restrict__ out, Tup<KW, PW>* const* __restrict__ peer_out = nullptr) {
+  static_assert(!PEER || CLAIM, "peer scatters claim their runs");
   using K = typename UW<KW>::T;
   using V = typename UW<PW>::T;
   using Tp = Tup<KW, PW>;
@@ -671,6 +680,7 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
   uint32_t* s_cur = s_dl + P4;                        // HBM write cursor per bucket
   uint32_t* s_wt = s_cur + P4;                        // warp totals
   uint64_t* bar = reinterpret_cast<uint64_t*>(s_wt + 64);
+  Tup<KW, PW>** s_out = reinterpret_cast<Tup<KW, PW>**>(bar + STAGES + 8);  // PEER: [P] destinations
 
   uint32_t seg, j, lo, hi;
   if constexpr (CLAIM) seg_chunk_tiles(m, blockIdx.x, (uint32_t)C::T, seg, j, lo, hi);
@@ -694,6 +704,7 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
       const size_t f = (size_t)(row0 + p) * m.cps + j;
       s_cur[p] = backward ? (f + 1 < nflat ? offsets[f + 1] : m.n) : offsets[f];
     }
+    if constexpr (PEER) s_out[p] = peer_out[p];
     s_cnt[p] = 0;
   }
   __syncthreads();
@@ -824,7 +835,13 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
       if constexpr (C::DST) return s_dst[i];
       else return s_dl[bucket_of(part_hash<KW, IDENT>(y.k), bf)] + i;
     };
-    if (full) {
+    if constexpr (PEER) {
+      for (uint32_t i = threadIdx.x; i < tn; i += NT) {
+        const Tp y = s_tile[i];
+        const uint32_t b = bucket_of(part_hash<KW, IDENT>(y.k), bf);
+        s_out[b][s_dl[b] + i] = y;
+      }
+    } else if (full) {
 #pragma unroll
       for (int u = 0; u < ITEMS; u++) {
         const uint32_t i = u * NT + threadIdx.x;
@@ -838,6 +855,7 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
       }
     }
   }
+  if constexpr (PEER) __threadfence_system();
 }
 
 // --------------------------------------------------------------------------

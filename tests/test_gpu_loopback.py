@@ -95,10 +95,11 @@ def test_route_segments_hold_their_destination(G, cfg, n):
             assert np.array_equal(got[0], want[0]) and np.array_equal(got[1], want[1])
 
 
+@pytest.mark.parametrize("peer", [False, True])
 @pytest.mark.parametrize("G", [2, 4, 8])
 @pytest.mark.parametrize("cfg,nr,ns", [("c1", 1 << 18, (1 << 18) + 4097), ("c3", 1 << 16, 1 << 18),
                                        ("dup", 6000, 7001), ("c5", 1 << 17, 1 << 19), ("mixed", 30011, 50021)])
-def test_loopback_join_vs_oracle(G, cfg, nr, ns):
+def test_loopback_join_vs_oracle(G, cfg, nr, ns, peer):
     wl = workload(cfg, nr, ns)
     kb, rb, sb = dtypes(wl)
     j = joiner(kb, rb, sb)
@@ -111,7 +112,7 @@ def test_loopback_join_vs_oracle(G, cfg, nr, ns):
     n = want["count"]
     out_r = torch.empty(max(n, 1), dtype=DT[rb], device="cuda")
     out_s = torch.empty(max(n, 1), dtype=DT[sb], device="cuda")
-    tot, per = j.loopback_join(r_sh, s_sh, out_r, out_s)
+    tot, per = j.loopback_join(r_sh, s_sh, out_r, out_s, peer=peer)
     got = dict(count=tot.match_count, sum_r=tot.sum_r_payload, sum_s=tot.sum_s_payload, checksum=tot.pair_checksum)
     assert got == {k: want[k] for k in got}
     assert tot.n_written == n
@@ -128,7 +129,8 @@ def test_loopback_join_vs_oracle(G, cfg, nr, ns):
         assert pd.r_local == int((dR == d).sum()) and pd.s_local == int((dS == d).sum())
 
 
-def test_loopback_ragged_and_empty_shards():
+@pytest.mark.parametrize("peer", [False, True])
+def test_loopback_ragged_and_empty_shards(peer):
     wl = datagen.make("c1", n_r=50000, n_s=70000)
     j = joiner(32, 32, 32)
     G = 4
@@ -137,21 +139,22 @@ def test_loopback_ragged_and_empty_shards():
     r_sh = [(cuda(wl.R.key[cr[g]:cr[g + 1]]), cuda(wl.R.payload[cr[g]:cr[g + 1]])) for g in range(G)]
     s_sh = [(cuda(wl.S.key[cs[g]:cs[g + 1]]), cuda(wl.S.payload[cs[g]:cs[g + 1]])) for g in range(G)]
     want = oracle.join(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload)
-    tot, per = j.loopback_join(r_sh, s_sh)
+    tot, per = j.loopback_join(r_sh, s_sh, peer=peer)
     assert (tot.match_count, tot.sum_r_payload, tot.sum_s_payload, tot.pair_checksum) == \
         (want["count"], want["sum_r"], want["sum_s"], want["checksum"])
     assert sum(p.r_local for p in per) == 50000 and sum(p.s_local for p in per) == 70000
 
 
 def test_loopback_results_identical_across_G():
-    """SURVEY §8.c.4 multi-GPU pin: the G = 1/2/4/8 results are bit-identical."""
+    """SURVEY §8.c.4 multi-GPU pin: the G = 1/2/4/8 results are bit-identical
+    (both exchange forms)."""
     wl = datagen.make("c2", n_r=1 << 19, n_s=1 << 19)
     j = joiner(32, 32, 32)
     res = set()
-    for G in (1, 2, 4, 8):
+    for G, peer in ((1, False), (2, False), (4, False), (8, False), (1, True), (2, True), (8, True), (16, True)):
         cut = [((1 << 19) * g) // G for g in range(G + 1)]
         sh = lambda rel: [(cuda(rel.key[cut[g]:cut[g + 1]]), cuda(rel.payload[cut[g]:cut[g + 1]])) for g in range(G)]
-        tot, _ = j.loopback_join(sh(wl.R), sh(wl.S))
+        tot, _ = j.loopback_join(sh(wl.R), sh(wl.S), peer=peer)
         res.add(tot.as_tuple())
     assert len(res) == 1
     assert next(iter(res))[0] == 1 << 19
