@@ -836,10 +836,16 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
       else return s_dl[bucket_of(part_hash<KW, IDENT>(y.k), bf)] + i;
     };
     if constexpr (PEER) {
-      for (uint32_t i = threadIdx.x; i < tn; i += NT) {
+      auto put = [&](uint32_t i) {
         const Tp y = s_tile[i];
         const uint32_t b = bucket_of(part_hash<KW, IDENT>(y.k), bf);
         s_out[b][s_dl[b] + i] = y;
+      };
+      if (full) {
+#pragma unroll
+        for (int u = 0; u < ITEMS; u++) put(u * NT + threadIdx.x);
+      } else {
+        for (uint32_t i = threadIdx.x; i < tn; i += NT) put(i);
       }
     } else if (full) {
 #pragma unroll
@@ -1002,7 +1008,15 @@ struct JnTable {
   const JnHead* head;
   uint32_t sbits;
   bool dup;                 // the chunk holds some key twice (bag semantics path)
+  uint32_t ep;              // stage epoch: a head is valid iff its high half == ep
 };
+
+// chain head of a slot: (epoch << 16) | tuple index; a head written in an
+// earlier stage (other epoch) reads as an empty chain, so the heads are never
+// reset between stages
+__device__ __forceinline__ uint32_t jn_head(JnHead hv, uint32_t ep) {
+  return (hv >> 16) == ep ? (hv & 0xFFFFu) : JN_NIL;
+}
 
 // Load U S tuples per consumer thread: j = base + u*256 + tid.
 template <int KW, int PSW, int U, int JN_CONSUMERS>
@@ -1027,7 +1041,7 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
 #pragma unroll
   for (int u = 0; u < U; u++) {
     const uint32_t j = base + u * JN_CONSUMERS + threadIdx.x;
-    e0[u] = j < s_hi ? t.head[jn_slot<KW>(x[u].k, t.sbits)] : JN_NIL;
+    e0[u] = j < s_hi ? jn_head(t.head[jn_slot<KW>(x[u].k, t.sbits)], t.ep) : JN_NIL;
   }
   uint32_t c[U], m[U];
 #pragma unroll
@@ -1039,20 +1053,43 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
     c[u] = 0;
     m[u] = JN_NIL;
     uint32_t e = e0[u];
-    while (true) {
-      while (e != JN_NIL && t.r[e].k != x[u].k) e = t.next[e];
-      const bool hit = e != JN_NIL;
-      if (!__any_sync(0xffffffffu, hit)) break;
-      if (hit) {
-        const int64_t pr = (int64_t)(PR)t.r[e].v, ps = (int64_t)(PS)x[u].v;
-        if (MAT && c[u] == 0) m[u] = e;
-        c[u]++;
+    if (!t.dup) {
+      // unique build side: walk to the first equal key (one 8/16-byte shared
+      // load per visited tuple gives key and payload), aggregate once
+      Tup<KW, PRW> y;
+      while (e != JN_NIL) {
+        y = t.r[e];
+        if (y.k == x[u].k) break;
+        e = t.next[e];
+      }
+      if (e != JN_NIL) {
+        const int64_t pr = (int64_t)(PR)y.v, ps = (int64_t)(PS)x[u].v;
+        if (MAT) m[u] = e;
+        c[u] = 1;
         acc.sr += (unsigned long long)pr;
         acc.ss += (unsigned long long)ps;
         acc.sx += pair_mix(pr, ps);
-        e = t.next[e];
       }
-      if (!t.dup) break;
+    } else {
+      while (true) {
+        Tup<KW, PRW> y;
+        while (e != JN_NIL) {
+          y = t.r[e];
+          if (y.k == x[u].k) break;
+          e = t.next[e];
+        }
+        const bool hit = e != JN_NIL;
+        if (!__any_sync(0xffffffffu, hit)) break;
+        if (hit) {
+          const int64_t pr = (int64_t)(PR)y.v, ps = (int64_t)(PS)x[u].v;
+          if (MAT && c[u] == 0) m[u] = e;
+          c[u]++;
+          acc.sr += (unsigned long long)pr;
+          acc.ss += (unsigned long long)ps;
+          acc.sx += pair_mix(pr, ps);
+          e = t.next[e];
+        }
+      }
     }
     acc.cnt += c[u];
   }
@@ -1164,6 +1201,9 @@ k_build_probe(JoinArgs a) {
     }
     asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
   }
+  // heads start in epoch 0, which no stage uses: every chain reads as empty
+  for (uint32_t i = threadIdx.x * 4; i < nslots; i += JN_THREADS * 4)
+    *reinterpret_cast<uint4*>(s_head + i) = make_uint4(0u, 0u, 0u, 0u);
   __syncthreads();
 
   if (warp == JN_CONSUMERS / 32) {
@@ -1218,19 +1258,20 @@ k_build_probe(JoinArgs a) {
     uint32_t sseq = 0;
     for (uint32_t stage = 0;; stage++) {
       const uint32_t bi = stage % NRB, ph = (stage / NRB) & 1;
-      // reset the heads (the previous stage's probe is complete: see the
-      // barrier at the end of the loop body), then wait for the R chunk
-      {
-        constexpr uint32_t HPV = 16 / sizeof(JnHead);  // heads per 16-byte store
-        constexpr uint32_t NILW = sizeof(JnHead) == 2 ? 0xFFFFFFFFu : JN_NIL;
-        for (uint32_t i = threadIdx.x * HPV; i < nslots; i += JN_CONSUMERS * HPV)
-          *reinterpret_cast<uint4*>(s_head + i) = make_uint4(NILW, NILW, NILW, NILW);
+      // stage epoch (1..65535): heads of other epochs read as empty chains,
+      // so the table needs no reset; every 65535 stages the heads are zeroed
+      // (epoch 0 is never used) -- the previous stage's probe is complete
+      // (barrier at the end of the loop body)
+      const uint32_t ep = stage % 65535u + 1u;
+      if (ep == 1u && stage > 0) {
+        for (uint32_t i = threadIdx.x * 4; i < nslots; i += JN_CONSUMERS * 4)
+          *reinterpret_cast<uint4*>(s_head + i) = make_uint4(0u, 0u, 0u, 0u);
+        consumer_sync<JN_CONSUMERS>();
       }
       mbar_wait(&full[bi], ph);
       const JnStage st = s_meta[bi];
       if (st.nr == JN_STOP) break;
       const TR* r = reinterpret_cast<const TR*>(ring + bi * RB + st.off);
-      consumer_sync<JN_CONSUMERS>();
       // ---- build (a11): chained table via atomicExch on the heads
       // the first S batch is loaded before the build so its latency hides
       // behind the table construction
@@ -1243,12 +1284,12 @@ k_build_probe(JoinArgs a) {
       if (PIPE && st.s_lo + BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, st.s_lo, st.s_hi, xs);
       if (!(a.dbg & 4u))
         for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
-          s_next[i] = (uint16_t)atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], i);
+          s_next[i] = (uint16_t)jn_head(atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], (ep << 16) | i), ep);
       consumer_sync<JN_CONSUMERS>();
       // ---- probe (a12): stream the S slice.  Bag semantics walk every chain
       // to its end; a caller-declared unique build side (HAPE_FLAG_R_UNIQUE, a
       // primary key) stops at the first match.
-      const JnTable<KW, PRW> tab{r, s_next, s_head, a.slot_bits, a.r_unique == 0};
+      const JnTable<KW, PRW> tab{r, s_next, s_head, a.slot_bits, a.r_unique == 0, ep};
       if constexpr (SR) {
         // staged S tiles: wait for the tile, copy this thread's tuples to
         // registers, release the tile (one arrival per warp), probe

@@ -10,4 +10,4 @@ for line in sys.stdin:
         continue
     st = d["roofline"]["stages"]
     print(d["config"]["workload"][:3], f"{d['ms_per_step']:.3f} ms", f"{d['value']/1e9:.1f} G/s",
-          " ".join(f"{k}={v['ms']:.3f}({v['frac']:.2f})" for k, v in st.items()))
+          " ".join(f"{k}={v['ms']:.3f}({v.get('frac', 0):.2f})" for k, v in st.items()))
