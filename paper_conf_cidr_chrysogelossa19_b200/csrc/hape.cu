@@ -150,6 +150,11 @@ static hape_status fail(hape_join* h, hape_status s, const char* fmt, ...) {
     CK(h, cudaGetLastError());                                                           \
   } while (0)
 
+static int env_int(const char* name, int dflt) {
+  const char* e = getenv(name);
+  return e ? atoi(e) : dflt;
+}
+
 static hape_status ensure(hape_join* h, DevBuf& b, size_t bytes) {
   if (bytes <= b.bytes) return HAPE_OK;
   if (b.p) {
@@ -401,8 +406,12 @@ static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, 
   CKS(smem_attr(h, k_scatter<KW, PW, AOS, C, IDENT, CLAIM>, 220 * 1024, attr_dev));
   const unsigned grid = m.nseg * m.cps;
   if (grid == 0) return HAPE_OK;
+  // warp-aggregated ranking: always for narrow fan-outs (the destination
+  // route, P <= 64: lanes share buckets), else HAPE_SC_AGG=1
+  static const uint32_t agg_env = (uint32_t)env_int("HAPE_SC_AGG", 0);
+  const uint32_t agg = agg_env || P <= 64;
   k_scatter<KW, PW, AOS, C, IDENT, CLAIM><<<grid, C::NT, smem, h->stream>>>(s.in, m, bf, P, offs,
-                                                                   static_cast<Tup<KW, PW>*>(out));
+                                                                   static_cast<Tup<KW, PW>*>(out), nullptr, agg);
   CK_LAUNCH(h);
   return HAPE_OK;
 }
@@ -467,8 +476,11 @@ static hape_status peer_scatter_t(hape_join* h, const Src& s, SegMap m, BitField
   CKS(smem_attr(h, kern, 220 * 1024, attr_dev));
   const unsigned grid = m.nseg * m.cps;
   if (grid == 0) return HAPE_OK;
+  // few destinations: the lanes of a warp share buckets -- warp-aggregated
+  // ranking (HAPE_SC_AGG_PEER=0 disables)
+  static const uint32_t agg = (uint32_t)env_int("HAPE_SC_AGG_PEER", 1);
   kern<<<grid, Cw::NT, smem, h->stream>>>(s.in, m, bf, P, offs, nullptr,
-                                         reinterpret_cast<Tup<KW, PW>* const*>(peers));
+                                         reinterpret_cast<Tup<KW, PW>* const*>(peers), agg);
   CK_LAUNCH(h);
   return HAPE_OK;
 }
@@ -492,10 +504,6 @@ static hape_status launch_peer_scatter(hape_join* h, int kw, const Src& s, SegMa
 // cannot keep a software-pipelined S batch in registers); the others read S
 // straight from HBM with a register-pipelined batch.  HAPE_JN_SU=0/1/2/4
 // forces the form, HAPE_JN_NRB / HAPE_JN_NSB the ring depths (tuning only).
-static int env_int(const char* name, int dflt) {
-  const char* e = getenv(name);
-  return e ? atoi(e) : dflt;
-}
 
 template <int KW, int PRW, int PSW, bool MAT, int SU, int NC = 256>
 static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* ctas_out) {

@@ -663,7 +663,8 @@ __device__ __forceinline__ void sc_issue(const PartIn& in, uint32_t t0, uint32_t
 template <int KW, int PW, bool AOS, class C, bool IDENT, bool CLAIM = false, bool PEER = false>
 __global__ void __launch_bounds__(C::NT, C::MINB)
 k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ offsets,
-          Tup<KW, PW>* __restrict__ out, Tup<KW, PW>* const* __restrict__ peer_out = nullptr) {
+          Tup<KW, PW>* __restrict__ out, Tup<KW, PW>* const* __restrict__ peer_out = nullptr,
+          uint32_t agg = 0) {
   static_assert(!PEER || CLAIM, "peer scatters claim their runs");
   using K = typename UW<KW>::T;
   using V = typename UW<PW>::T;
@@ -733,22 +734,42 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
     Tp x[ITEMS];
     uint32_t br[ITEMS];
     const bool full = tn == (uint32_t)T;
+    // agg (skewed inputs): lanes of a warp that share a bucket rank through
+    // one leader atomic (__match_any_sync) instead of
+    // serialising on the same shared-memory word
+    auto rank_agg = [&](uint32_t b, uint32_t mask) -> uint32_t {
+      const uint32_t peers = __match_any_sync(mask, b);
+      const int leader = __ffs(peers) - 1;
+      uint32_t base = 0;
+      if (lane == leader) base = atomicAdd(&s_cnt[b], (uint32_t)__popc(peers));
+      base = __shfl_sync(peers, base, leader);
+      return base + (uint32_t)__popc(peers & ((1u << lane) - 1u));
+    };
     if (full) {
 #pragma unroll
       for (int u = 0; u < ITEMS; u++) x[u] = load(u * NT + threadIdx.x);
+      if (agg) {
 #pragma unroll
-      for (int u = 0; u < ITEMS; u++) {
-        const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
-        br[u] = (b << 16) | atomicAdd(&s_cnt[b], 1u);
+        for (int u = 0; u < ITEMS; u++) {
+          const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
+          br[u] = (b << 16) | rank_agg(b, 0xffffffffu);
+        }
+      } else {
+#pragma unroll
+        for (int u = 0; u < ITEMS; u++) {
+          const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
+          br[u] = (b << 16) | atomicAdd(&s_cnt[b], 1u);
+        }
       }
     } else {
 #pragma unroll
       for (int u = 0; u < ITEMS; u++) {
         const uint32_t i = u * NT + threadIdx.x;
+        const uint32_t vm = __ballot_sync(0xffffffffu, i < tn);
         if (i < tn) {
           x[u] = load(i);
           const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
-          br[u] = (b << 16) | atomicAdd(&s_cnt[b], 1u);
+          br[u] = (b << 16) | (agg ? rank_agg(b, vm) : atomicAdd(&s_cnt[b], 1u));
         }
       }
     }
