@@ -9,6 +9,9 @@ Contents
   join(...)        -- oracle.c: single-threaded sort-merge computing the plain
                       definition of the §6.2 micro-benchmark result
                       (PAPER.md P789-794), see oracle.c's header.
+  join_sharded(...) -- the same oracle on T host threads:
+                      R and S split by key into T shards (equal keys share a
+                      shard), one oracle.c join per shard, sums mod 2^64.
   mix / fmix64     -- numpy re-statement of the pair-checksum term (DESIGN.md
                       reading R10); pinned by published splitmix64 vectors.
   partition.py     -- the partition function h and its bit fields (DESIGN.md
@@ -145,3 +148,37 @@ def u64sum(x: np.ndarray) -> int:
 
 def threads_used() -> int:
     return 1
+
+
+def host_cores() -> int:
+    try:
+        return len(os.sched_getaffinity(0))
+    except Exception:
+        return os.cpu_count() or 1
+
+
+def join_sharded(rk, rp, sk, sp, threads: int = 0) -> dict:
+    """SURVEY §8.d.6's T-core variant of the oracle (count and sums only):
+    shard s gets the tuples whose key k has (k mod T) == s -- a plain
+    function of the key, so equal keys meet in one shard and the shard
+    results add up to the whole join -- and each shard runs join() on its
+    own thread (the C call releases the GIL).  T = host cores by default."""
+    from concurrent.futures import ThreadPoolExecutor
+    T = threads or host_cores()
+    rk, rp, sk, sp = (_np(x) for x in (rk, rp, sk, sp))
+
+    def shard(i):
+        # every thread selects its own shard (numpy releases the GIL on the
+        # array passes, so the selection runs in parallel too)
+        if T == 1:
+            return join(rk, rp, sk, sp)
+        mr = (rk.astype(np.int64) % T) == i
+        ms = (sk.astype(np.int64) % T) == i
+        return join(rk[mr], rp[mr], sk[ms], sp[ms])
+
+    with ThreadPoolExecutor(max_workers=T) as ex:
+        parts = list(ex.map(shard, range(T)))
+    M = (1 << 64) - 1
+    return dict(count=sum(p["count"] for p in parts), sum_r=sum(p["sum_r"] for p in parts) & M,
+                sum_s=sum(p["sum_s"] for p in parts) & M, checksum=sum(p["checksum"] for p in parts) & M,
+                threads=T)

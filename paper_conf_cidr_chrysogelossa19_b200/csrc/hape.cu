@@ -513,7 +513,7 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
   JoinArgs a = a_in;
   static const int nrb_env = env_int("HAPE_JN_NRB", 0), nsb_env = env_int("HAPE_JN_NSB", 0);
   a.nsb = SR ? (uint32_t)std::min(8, std::max(2, nsb_env ? nsb_env : (SU >= 4 ? 3 : 2))) : 0u;
-  a.nrb = SR ? (uint32_t)std::min(2, std::max(1, nrb_env ? nrb_env : 2)) : 2u;
+  a.nrb = (uint32_t)std::min(2, std::max(1, nrb_env ? nrb_env : 2));
   static uint64_t attr_dev = 0;
   CKS(smem_attr(h, kern, 200 * 1024, attr_dev));
   auto occ = [&](uint32_t sb, uint32_t nrb, int* per_sm) -> hape_status {
@@ -525,9 +525,11 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
   };
   int per_sm = 0;
   CKS(occ(a.slot_bits, a.nrb, &per_sm));
-  // a single R buffer when the second one would cost a CTA per SM (SR: the
-  // other resident CTAs cover the R load at a stage boundary)
-  if (SR && !nrb_env && a.nrb == 2) {
+  // a single R buffer when the second one would cost a CTA per SM (the
+  // other resident CTAs cover the R load at a stage boundary); the direct
+  // form only with HAPE_JN_NRB1=1 (A/B)
+  static const int nrb1_direct = env_int("HAPE_JN_NRB1", 0);
+  if ((SR || nrb1_direct) && !nrb_env && a.nrb == 2) {
     int p1 = 0;
     CKS(occ(a.slot_bits, 1, &p1));
     if (p1 > per_sm) { a.nrb = 1; per_sm = p1; }

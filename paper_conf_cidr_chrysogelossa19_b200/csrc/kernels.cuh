@@ -1196,7 +1196,7 @@ k_build_probe(JoinArgs a) {
   extern __shared__ __align__(128) unsigned char smem[];
   const uint32_t RB = (uint32_t)join_ring_bytes<KW, PRW>(a.cap);
   constexpr uint32_t SB = SR ? (uint32_t)join_stile_bytes<KW, PSW, SR ? SU : 1, JN_CONSUMERS>() : 0u;
-  const uint32_t NRB = SR ? a.nrb : 2u, NSB = SR ? a.nsb : 0u;
+  const uint32_t NRB = a.nrb, NSB = SR ? a.nsb : 0u;
   unsigned char* ring = smem;                                           // [NRB][RB]
   unsigned char* sring = smem + NRB * RB;                               // [NSB][SB]
   uint16_t* s_next = reinterpret_cast<uint16_t*>(sring + NSB * SB);

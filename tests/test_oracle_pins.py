@@ -67,6 +67,25 @@ def test_murmur3_fmix32_published_vectors(golden_dir):
         assert int(partition.fmix32(k)[0]) == int(want, 16)
 
 
+def test_mix_pinned_by_published_splitmix64(golden_dir):
+    """The pair-checksum term itself (not a restatement of it): with
+    mix(p, q) = fmix64(p*phi + q) (R10), mix(k, 0) = fmix64(k*phi)
+    is the k-th published splitmix64 seed-0 output, and so is
+    mix(k - 1, phi as int64) -- pinning the multiplier and the additive q
+    term (a dropped term, a swapped operand or a missing sign extension of q
+    breaks one of the two)."""
+    g = json.load(open(os.path.join(golden_dir, "hash_vectors.json")))
+    want = [int(v, 16) for v in g["splitmix64_seed0"]]
+    phi_i64 = 0x9E3779B97F4A7C15 - (1 << 64)          # negative as int64: sign extension matters
+    for k, w in zip((1, 2, 3), want):
+        assert oracle.mix_scalar(k, 0) == w
+        assert oracle.mix_scalar(k - 1, phi_i64) == w
+        assert int(oracle.mix(np.array([k], np.int64), np.array([0], np.int64))[0]) == w
+        assert int(oracle.mix(np.array([k - 1], np.int64), np.array([phi_i64], np.int64))[0]) == w
+        # 32-bit payloads: p = k fits; the q term through a sign-extended int32
+    assert int(oracle.mix(np.array([1], np.int32), np.array([0], np.int32))[0]) == want[0]
+
+
 def test_mix_orientation_and_sign_extension():
     # mix is orientation-sensitive and sign-extends 32-bit payloads
     assert oracle.mix_scalar(1, 2) != oracle.mix_scalar(2, 1)
@@ -195,3 +214,16 @@ def test_oracle_vs_provenance(cfg, nr, ns):
     assert np.array_equal(got["pairs"][0], exp_pairs[0])
     assert np.array_equal(got["pairs"][1], exp_pairs[1])
     assert got["count"] == ns  # closed form (P793-794)
+
+
+@pytest.mark.parametrize("threads", [1, 3, 8])
+def test_sharded_oracle_equals_oracle(threads):
+    """SURVEY §8.d.6's T-thread oracle adds up to the single-thread one."""
+    rng = np.random.default_rng(31 + threads)
+    rk = rng.integers(-500, 500, 20000).astype(np.int64)
+    sk = rng.integers(-600, 600, 30000).astype(np.int64)
+    rp = rng.integers(-2**40, 2**40, 20000).astype(np.int64)
+    sp = rng.integers(-2**40, 2**40, 30000).astype(np.int32)
+    want = oracle.join(rk, rp, sk, sp)
+    got = oracle.join_sharded(rk, rp, sk, sp, threads=threads)
+    assert {k: got[k] for k in want} == want and got["threads"] == threads
