@@ -10,7 +10,8 @@ import ctypes
 import os
 
 _PKG = os.path.dirname(os.path.abspath(__file__))
-LIB_PATH = os.path.join(_PKG, "libhape.so")
+# HAPE_LIB: an A/B variant built by build.py --out (tuning only)
+LIB_PATH = os.environ.get("HAPE_LIB") or os.path.join(_PKG, "libhape.so")
 
 HAPE_OK = 0
 HAPE_ERR_INVALID_ARG = 1
