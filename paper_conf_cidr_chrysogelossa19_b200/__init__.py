@@ -110,7 +110,7 @@ class RadixJoin:
     def __init__(self, key_dtype=None, r_payload_dtype=None, s_payload_dtype=None, device: int = 0,
                  radix_passes: int = 0, radix_bits=(0, 0), identity: bool = False,
                  max_r: int = 0, max_s: int = 0, world_size: int = 1, rank: int = 0,
-                 nccl_comm=None, stream=None, r_unique: bool = False):
+                 nccl_comm=None, stream=None, r_unique: bool = False, linked: bool = False):
         import torch
         key_dtype = key_dtype or torch.int32
         cfg = hape_join_config()
@@ -123,7 +123,7 @@ class RadixJoin:
         cfg.part_fn = HAPE_PART_IDENTITY if identity else HAPE_PART_HASH
         cfg.max_r, cfg.max_s = max_r, max_s
         cfg.world_size, cfg.rank = world_size, rank
-        cfg.flags = _lib.HAPE_FLAG_R_UNIQUE if r_unique else 0
+        cfg.flags = (_lib.HAPE_FLAG_R_UNIQUE if r_unique else 0) | (_lib.HAPE_FLAG_LINKED if linked else 0)
         cfg.nccl_comm = nccl_comm.value if isinstance(nccl_comm, ctypes.c_void_p) else nccl_comm
         # the library enqueues on the caller's stream (inputs must be ready on
         # it): default to torch's current stream on the device

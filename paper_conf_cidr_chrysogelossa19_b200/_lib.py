@@ -28,6 +28,7 @@ HAPE_PART_IDENTITY = 1
 HAPE_MEM_DEVICE = 0
 HAPE_MEM_HOST = 1
 HAPE_FLAG_R_UNIQUE = 1
+HAPE_FLAG_LINKED = 2
 
 STAGES = ["h2d", "devpart", "exchange", "hist1", "scan1", "scatter1", "hist2", "scan2",
           "scatter2", "worklist", "build_probe", "np_build", "np_probe", "finalize", "host_part", "total"]

@@ -101,6 +101,7 @@ struct hape_join {
   bool p2p_failed = false;              // IPC unavailable: NCCL send/recv from then on
   // hape_debug_loopback_join (peer form): one receive buffer per simulated rank
   DevBuf lb_rx[2][64];
+  DevBuf lbuf[2];                       // HAPE_FLAG_LINKED: buffer directory, owner, chain index
   uint32_t xchg_path = 0;               // last call: 0 none, 1 NCCL send/recv, 2 peer scatter
   bool peer_tab_dirty = false;          // peer_tab holds the loopback's table
 };
@@ -305,10 +306,17 @@ static hape_status launch_hist(hape_join* h, int kw, const Src& s, SegMap m, Bit
 // Two-pass plans with B1 + B2 <= 16 count both passes' buckets in one read of
 // the keys (k_hist_joint) and run pass 2 as a claiming scatter.  HAPE_JOINT=0
 // forces the separate pass-2 histogram (tests compare both forms).
-static bool use_joint(const hape_plan& pl) {
+// HAPE_FLAG_LINKED: two-pass plans run pass 1 as the paper's single-scan
+// linked-buffer partitioning (no histogram before it; pass 2 reads the
+// chains and counts its own buckets)
+static bool use_linked(const hape_join* h, const hape_plan& pl) {
+  return (h->cfg.flags & HAPE_FLAG_LINKED) && pl.passes == 2;
+}
+
+static bool use_joint(const hape_join* h, const hape_plan& pl) {
   static const int env = [] { const char* e = getenv("HAPE_JOINT"); return e ? atoi(e) : 1; }();
-  return env != 0 && pl.passes == 2 && pl.bits[0] + pl.bits[1] <= 16 && pl.bits[0] + pl.bits[1] >= 6 &&
-         pl.bits[1] >= 1;
+  return env != 0 && !use_linked(h, pl) && pl.passes == 2 && pl.bits[0] + pl.bits[1] <= 16 &&
+         pl.bits[0] + pl.bits[1] >= 6 && pl.bits[1] >= 1;
 }
 
 // Plans the joint histogram cannot count (one pass, or B1 + B2 > 16) still
@@ -317,9 +325,9 @@ static bool use_joint(const hape_plan& pl) {
 // and claim cursors, and the scatter claims runs from the cursors (the
 // per-CTA offset form costs 0.38-0.49 of the HBM roofline at 2^20 buckets:
 // runs of a few tuples per CTA chunk).  HAPE_CLAIM=0 keeps the per-CTA form.
-static bool use_claim(const hape_plan& pl) {
+static bool use_claim(const hape_join* h, const hape_plan& pl) {
   static const int env = [] { const char* e = getenv("HAPE_CLAIM"); return e ? atoi(e) : 1; }();
-  return env != 0 && !use_joint(pl);
+  return (env != 0 || use_linked(h, pl)) && !use_joint(h, pl);
 }
 
 static uint32_t joint_grid(const hape_join* h, uint32_t nchunks) {
@@ -398,23 +406,52 @@ static hape_status launch_scan(hape_join* h, SegMap m, uint32_t P, uint32_t* his
   return HAPE_OK;
 }
 
-template <int KW, int PW, bool AOS, class C, bool IDENT, bool CLAIM>
+template <int KW, int PW, bool AOS, class C, bool IDENT, bool CLAIM, bool LINKED = false>
 static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* offs,
-                             void* out) {
-  const size_t smem = ScLayout<KW, PW, AOS, C>::bytes(P);
+                             void* out, const LinkMap* lk = nullptr) {
+  const size_t smem = ScLayout<KW, PW, AOS, C>::bytes(P, false, LINKED);
   static uint64_t attr_dev = 0;
-  CKS(smem_attr(h, k_scatter<KW, PW, AOS, C, IDENT, CLAIM>, 220 * 1024, attr_dev));
+  auto kern = k_scatter<KW, PW, AOS, C, IDENT, CLAIM, false, LINKED>;
+  CKS(smem_attr(h, kern, 220 * 1024, attr_dev));
   const unsigned grid = m.nseg * m.cps;
   if (grid == 0) return HAPE_OK;
   // warp-aggregated ranking: always for narrow fan-outs (the destination
   // route, P <= 64: lanes share buckets), else HAPE_SC_AGG=1
   static const uint32_t agg_env = (uint32_t)env_int("HAPE_SC_AGG", 0);
   const uint32_t agg = agg_env || P <= 64;
-  k_scatter<KW, PW, AOS, C, IDENT, CLAIM><<<grid, C::NT, smem, h->stream>>>(s.in, m, bf, P, offs,
-                                                                   static_cast<Tup<KW, PW>*>(out), nullptr, agg);
+  kern<<<grid, C::NT, smem, h->stream>>>(s.in, m, bf, P, offs, static_cast<Tup<KW, PW>*>(out), nullptr, agg,
+                                         lk ? *lk : LinkMap{});
   CK_LAUNCH(h);
   return HAPE_OK;
 }
+
+// pass 1 of the linked-buffer partitioning (k_scatter LINKED), default shapes
+template <int KW, int PW, bool AOS>
+static hape_status scatter_linked_v(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, void* out,
+                                    const LinkMap& lk) {
+  using C = typename std::conditional<KW + PW <= 8, ScCfg<512, 13, 2, 2>, ScCfg<384, 9, 2, 2>>::type;
+  if (h->cfg.part_fn == HAPE_PART_IDENTITY)
+    return scatter_t<KW, PW, AOS, C, true, true, true>(h, s, m, bf, P, lk.cnt, out, &lk);
+  return scatter_t<KW, PW, AOS, C, false, true, true>(h, s, m, bf, P, lk.cnt, out, &lk);
+}
+
+static hape_status launch_scatter_linked(hape_join* h, int kw, const Src& s, SegMap m, BitField bf, uint32_t P,
+                                         void* out, const LinkMap& lk) {
+  const int pw = s.pw;
+#define HAPE_SCL(AOS)                                                                  \
+  if (kw == 4 && pw == 4) return scatter_linked_v<4, 4, AOS>(h, s, m, bf, P, out, lk); \
+  if (kw == 4) return scatter_linked_v<4, 8, AOS>(h, s, m, bf, P, out, lk);            \
+  if (pw == 4) return scatter_linked_v<8, 4, AOS>(h, s, m, bf, P, out, lk);            \
+  return scatter_linked_v<8, 8, AOS>(h, s, m, bf, P, out, lk);
+  if (s.aos) { HAPE_SCL(true) } else { HAPE_SCL(false) }
+#undef HAPE_SCL
+}
+
+// linked-buffer geometry: buffers of two default scatter tiles (pass 2 reads
+// whole tiles), a dense directory row of kmax entries per pass-1 bucket
+static uint32_t lb_buf(size_t tb) { return tb <= 8 ? 2u * 512u * 13u : 2u * 384u * 9u; }
+static uint64_t lb_nbuf(uint64_t n, size_t tb, uint32_t P1) { return (n + lb_buf(tb) - 1) / lb_buf(tb) + P1; }
+static uint64_t lb_kmax(uint64_t n, size_t tb) { return (n + lb_buf(tb) - 1) / lb_buf(tb) + 1; }
 
 // scatter shape per tuple width (measured best of the ScCfg sweep);
 // (the destination-table variant ScCfg<..., DST=true> is no longer dispatched)
@@ -480,7 +517,7 @@ static hape_status peer_scatter_t(hape_join* h, const Src& s, SegMap m, BitField
   // ranking (HAPE_SC_AGG_PEER=0 disables)
   static const uint32_t agg = (uint32_t)env_int("HAPE_SC_AGG_PEER", 1);
   kern<<<grid, Cw::NT, smem, h->stream>>>(s.in, m, bf, P, offs, nullptr,
-                                         reinterpret_cast<Tup<KW, PW>* const*>(peers), agg);
+                                         reinterpret_cast<Tup<KW, PW>* const*>(peers), agg, LinkMap{});
   CK_LAUNCH(h);
   return HAPE_OK;
 }
@@ -687,6 +724,7 @@ struct SideLayout {            // per relation
   // [Q] (zeroed), part the per-CTA 16-bit joint histograms [nparts][Q]
   size_t part = 0;
   uint32_t nparts = 0;
+  size_t lpool = 0;          // linked pass 1: buffers handed out (zeroed)
 };
 
 struct CallLayout {
@@ -709,16 +747,17 @@ static CallLayout layout_for(const hape_join* h, const hape_plan& pl, uint64_t n
   L.ctrs = cv.take(8);
   const uint64_t ns[2] = {n_r, n_s};
   for (int s = 0; s < 2; s++) {
-    L.side[s].rowsum1 = cv.take(P1 * 4);
+    L.side[s].rowsum1 = cv.take(P1 * 4);   // (linked pass 1: the buckets' claim counters)
     if (pl.passes == 2) L.side[s].rowsum2 = cv.take(Q * 4);
+    if (use_linked(h, pl)) L.side[s].lpool = cv.take(8);
   }
   L.zero_hi = cv.off;
   for (int s = 0; s < 2; s++) {
     SideLayout& S = L.side[s];
     S.cps1 = cps_for(h, ns[s], 1);
-    S.hist1 = cv.take(P1 * (use_joint(pl) || use_claim(pl) ? 1 : S.cps1) * 4);  // joint / claim: pass-1 cursors
+    S.hist1 = cv.take(P1 * (use_joint(h, pl) || use_claim(h, pl) ? 1 : S.cps1) * 4);  // joint / claim: pass-1 cursors
     S.bounds1 = cv.take((P1 + 1) * 4);
-    if (pl.passes == 2 && use_joint(pl)) {
+    if (pl.passes == 2 && use_joint(h, pl)) {
       S.cps2 = cps_for(h, ns[s], (uint32_t)P1);
       S.hist2 = cv.take(Q * 4);
       S.bounds2 = cv.take((Q + 1) * 4);
@@ -726,7 +765,7 @@ static CallLayout layout_for(const hape_join* h, const hape_plan& pl, uint64_t n
       S.part = cv.take((size_t)S.nparts * Q * 2);
     } else if (pl.passes == 2) {
       S.cps2 = cps_for(h, ns[s], (uint32_t)P1);
-      S.hist2 = cv.take(Q * (use_claim(pl) ? 1 : S.cps2) * 4);
+      S.hist2 = cv.take(Q * (use_claim(h, pl) ? 1 : S.cps2) * 4);
       S.bounds2 = cv.take((Q + 1) * 4);
     }
   }
@@ -773,8 +812,8 @@ static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const
   // scatters claim; hist2 / scan2 are empty.  Workspace reuse: hist1 / hist2
   // hold the pass-1 / pass-2 cursors, rowsum1 the row totals, rowsum2 the
   // spilled counts (both zeroed per call).
-  const bool joint = use_joint(pl);
-  const bool claim = use_claim(pl);
+  const bool joint = use_joint(h, pl);
+  const bool claim = use_claim(h, pl);
   // claim form: totals -> cursors (the scan reads them as a one-CTA histogram)
   auto totals_scan = [&](SegMap m, uint32_t P, size_t cur_off, size_t rs_off, size_t bnd_off) {
     const size_t rows = (size_t)m.nseg * P;
@@ -822,7 +861,45 @@ static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const
     return launch_scatter(h, kw, s2[s], m2[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), io[s].p2,
                           joint || claim);
   };
-  if (side1_ready) {
+  if (use_linked(h, pl)) {
+    // the single-scan form (P593-597): pass 1 claims into buffer chains with
+    // no histogram before it; pass 2 reads the chains, counts its buckets
+    // (totals), and claims into the dense pass-2 layout.  Stage marks:
+    // hist1 = directory reset, scatter1 = linked scatter + pass-1 bounds.
+    LinkMap lk[2];
+    SegMap mb[2];
+    for (int s = 0; s < nside; s++) {
+      const uint64_t n = io[s].in.n;
+      const size_t tb = tup_bytes(kw, io[s].in.pw);
+      const uint32_t B = lb_buf(tb);
+      const uint64_t nb = lb_nbuf(n, tb, P1), km = lb_kmax(n, tb);
+      const size_t dir_b = (size_t)P1 * km * 4;
+      CKS(ensure(h, h->lbuf[s], dir_b + 2 * nb * 4 + 64));
+      uint32_t* dir = static_cast<uint32_t*>(h->lbuf[s].p);
+      uint32_t* owner = dir + (size_t)P1 * km;
+      uint32_t* kidx = owner + nb;
+      lk[s] = LinkMap{at<uint32_t>(h, L.side[s].rowsum1), at<uint32_t>(h, L.side[s].lpool), dir, owner, kidx,
+                      (uint32_t)km, B};
+      mb[s] = SegMap{nullptr, (uint32_t)nb, 1u, (uint32_t)n, owner, kidx, lk[s].cnt, lk[s].pool, B};
+      s2[s] = Src{PartIn{nullptr, nullptr, io[s].p1}, true, (uint32_t)n, io[s].in.pw};
+    }
+    for (int s = 0; s < nside; s++) {
+      if (s == 1 && side1_ready) CK(h, cudaStreamWaitEvent(h->stream, side1_ready, 0));
+      if (s == 0) mark(h, HAPE_STAGE_HIST1);
+      CK(h, cudaMemsetAsync(lk[s].dir, 0, (size_t)P1 * lk[s].kmax * 4, h->stream));
+      if (s == 0) mark(h, HAPE_STAGE_SCATTER1);
+      CKS(launch_scatter_linked(h, kw, io[s].in, m1[s], bf1, P1, io[s].p1, lk[s]));
+      CKS(totals_scan(m1[s], P1, L.side[s].hist1, L.side[s].rowsum1, L.side[s].bounds1));
+    }
+    mark(h, HAPE_STAGE_HIST2);
+    for (int s = 0; s < nside; s++)
+      CKS(launch_hist(h, kw, s2[s], mb[s], bf2, P2, nullptr, at<uint32_t>(h, L.side[s].rowsum2)));
+    mark(h, HAPE_STAGE_SCAN2);
+    for (int s = 0; s < nside; s++) CKS(scan2(s));
+    mark(h, HAPE_STAGE_SCATTER2);
+    for (int s = 0; s < nside; s++)
+      CKS(launch_scatter(h, kw, s2[s], mb[s], bf2, P2, at<uint32_t>(h, L.side[s].hist2), io[s].p2, true));
+  } else if (side1_ready) {
     for (int s = 0; s < nside; s++) {
       if (s == 1) CK(h, cudaStreamWaitEvent(h->stream, side1_ready, 0));
       if (s == 0) mark(h, HAPE_STAGE_HIST1);
@@ -1160,6 +1237,12 @@ static void stage_times(hape_join* h, hape_join_result* res) {
   (void)cudaGetLastError();
 }
 
+// pass-1 output bytes: the relation, or (linked pass 1) its buffer pool
+static size_t ping_bytes(const hape_join* h, const hape_plan& pl, uint64_t n, size_t tb) {
+  if (use_linked(h, pl)) return (size_t)lb_nbuf(n, tb, 1u << pl.bits[0]) * lb_buf(tb) * tb + 16;
+  return (size_t)n * tb + 16;
+}
+
 // ---------------------------------------------------------------------------
 // the local join (a6-a13 over one GPU's share): plan, radix passes, work
 // list, build+probe, local result D2H into h_res[0..5] (acc[4], out_ctr,
@@ -1187,7 +1270,7 @@ static hape_status local_join(hape_join* h, const Src loc_in[2], const MatOut& m
   const uint64_t n_loc[2] = {loc[0].n, loc[1].n};
   const int pw[2] = {prw, psw};
   for (int s = 0; s < 2; s++) {
-    CKS(ensure(h, h->ping[s], n_loc[s] * tup_bytes(kw, pw[s]) + 16));
+    CKS(ensure(h, h->ping[s], ping_bytes(h, pl, n_loc[s], tup_bytes(kw, pw[s]))));
     if (pl.passes == 2) CKS(ensure(h, h->pong[s], n_loc[s] * tup_bytes(kw, pw[s]) + 16));
   }
   const uint32_t Q = 1u << (pl.bits[0] + (pl.passes == 2 ? pl.bits[1] : 0));
@@ -1737,7 +1820,7 @@ hape_status hape_join_create(const hape_join_config* cfg, hape_join** out_handle
   if (cfg->rank < 0 || cfg->rank >= world) return HAPE_ERR_INVALID_ARG;
   if (world > 1 && !cfg->nccl_comm) return HAPE_ERR_INVALID_ARG;
   if (cfg->device < 0) return HAPE_ERR_INVALID_ARG;
-  if (cfg->flags & ~HAPE_FLAG_R_UNIQUE) return HAPE_ERR_INVALID_ARG;
+  if (cfg->flags & ~(HAPE_FLAG_R_UNIQUE | HAPE_FLAG_LINKED)) return HAPE_ERR_INVALID_ARG;
   int ndev = 0;
   if (cudaGetDeviceCount(&ndev) != cudaSuccess || cfg->device >= ndev) {
     (void)cudaGetLastError();
@@ -1828,6 +1911,8 @@ hape_status hape_join_destroy(hape_join* h) {
       if (b.p) cudaFree(b.p);
   }
   if (h->peer_tab.p) cudaFree(h->peer_tab.p);
+  for (auto& b : h->lbuf)
+    if (b.p) cudaFree(b.p);
   if (h->xipc.p) cudaFree(h->xipc.p);
   if (h->h_x) cudaFreeHost(h->h_x);
   if (h->xb.p) cudaFree(h->xb.p);
@@ -1900,7 +1985,7 @@ hape_status hape_debug_partition(hape_join* h, const hape_relation* rel, int is_
   CKS(stage_in(h, rel, kw, pw, h->stage[0], h->stage[1], &in));
   const CallLayout L = layout_for(h, pl, rel->n, rel->n);
   CKS(ensure(h, h->small, L.total));
-  CKS(ensure(h, h->ping[0], rel->n * tup_bytes(kw, pw) + 16));
+  CKS(ensure(h, h->ping[0], ping_bytes(h, pl, rel->n, tup_bytes(kw, pw))));
   CKS(ensure(h, h->pong[0], rel->n * tup_bytes(kw, pw) + 16));
   CK(h, cudaMemsetAsync(at<char>(h, L.zero_lo), 0, L.zero_hi - L.zero_lo, h->stream));
   PassIO io[2];

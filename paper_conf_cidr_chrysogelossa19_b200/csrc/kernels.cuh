@@ -75,15 +75,51 @@ __device__ __forceinline__ uint64_t pair_mix(int64_t p, int64_t q) {
 // segment -> CTA chunk mapping, shared by k_hist and k_scatter of one pass
 // (the offsets are only right if both kernels see identical chunks)
 // --------------------------------------------------------------------------
+// Linked-buffer chains (the paper's single-scan partitioning, P593-597;
+// SURVEY §8.f NEXT-2): bucket b's tuples sit in a chain of fixed-size
+// buffers of `buf` tuples, buffer k of the chain at physical id dir[b*kmax+k]-1;
+// owner[id] / kidx[id] invert it, cnt[b] is the bucket's tuple count, *pool
+// the number of buffers handed out.
+struct LinkMap {
+  uint32_t* cnt;
+  uint32_t* pool;
+  uint32_t* dir;
+  uint32_t* owner;
+  uint32_t* kidx;
+  uint32_t kmax;
+  uint32_t buf;
+};
+
 struct SegMap {
   const uint32_t* bounds;  // nseg+1 segment bounds (device) or nullptr: one segment [0, n)
   uint32_t nseg;
   uint32_t cps;            // CTAs per segment
   uint32_t n;
+  // chained input (a pass reading linked buffers): CTA j reads buffer j,
+  // its segment is the buffer's owner; nseg = upper bound of buffers
+  const uint32_t* owner = nullptr;
+  const uint32_t* kidx = nullptr;
+  const uint32_t* cnt = nullptr;
+  const uint32_t* pool = nullptr;
+  uint32_t buf = 0;
 };
+
+// buffer j of a chained input: segment and physical range (empty when j is
+// beyond the buffers handed out)
+__device__ __forceinline__ void buf_chunk(const SegMap& m, uint32_t cta, uint32_t& seg, uint32_t& j,
+                                          uint32_t& lo, uint32_t& hi) {
+  j = 0;
+  if (cta >= *m.pool) { seg = 0; lo = hi = 0; return; }
+  seg = m.owner[cta];
+  const uint32_t k = m.kidx[cta];
+  const uint32_t fill = min(m.buf, m.cnt[seg] - k * m.buf);
+  lo = cta * m.buf;
+  hi = lo + fill;
+}
 
 __device__ __forceinline__ void seg_chunk(const SegMap& m, uint32_t cta, uint32_t& seg,
                                           uint32_t& j, uint32_t& lo, uint32_t& hi) {
+  if (m.owner) { buf_chunk(m, cta, seg, j, lo, hi); return; }
   seg = cta / m.cps;
   j = cta - seg * m.cps;
   uint32_t b = m.bounds ? m.bounds[seg] : 0u;
@@ -98,6 +134,7 @@ __device__ __forceinline__ void seg_chunk(const SegMap& m, uint32_t cta, uint32_
 // the partial-tile path.
 __device__ __forceinline__ void seg_chunk_tiles(const SegMap& m, uint32_t cta, uint32_t T, uint32_t& seg,
                                                 uint32_t& j, uint32_t& lo, uint32_t& hi) {
+  if (m.owner) { buf_chunk(m, cta, seg, j, lo, hi); return; }
   seg = cta / m.cps;
   j = cta - seg * m.cps;
   const uint32_t b = m.bounds ? m.bounds[seg] : 0u;
@@ -618,9 +655,10 @@ struct ScLayout {
   static constexpr size_t RP = AOS ? 0 : (size_t)T * PW + 32;
   static constexpr size_t RAW0 = (RK + RP + 15) / 16 * 16;
   static constexpr size_t RAW = RAW0 > (size_t)T * sizeof(Tp) ? RAW0 : (size_t)T * sizeof(Tp);
-  static __host__ __device__ constexpr size_t bytes(uint32_t P, bool peer = false) {
+  static __host__ __device__ constexpr size_t bytes(uint32_t P, bool peer = false, bool linked = false) {
     return C::STAGES * RAW + (C::DST ? (size_t)T * 4 : 0) + (size_t)((P + 3) & ~3u) * 16 + 64 * 4 +
-           C::STAGES * 8 + 64 + (peer ? (size_t)((P + 1) & ~1u) * 8 : 0);
+           C::STAGES * 8 + 64 + (peer ? (size_t)((P + 1) & ~1u) * 8 : 0) +
+           (linked ? (size_t)((P + 3) & ~3u) * 8 : 0);
   }
 };
 
@@ -660,12 +698,26 @@ __device__ __forceinline__ void sc_issue(const PartIn& in, uint32_t t0, uint32_t
 // peers' memory straight from the staging tile -- no send buffer, no separate
 // transfer.  Every thread fences at system scope before exiting, so the
 // stores are visible to the peers once their stream-ordered barrier passes.
-template <int KW, int PW, bool AOS, class C, bool IDENT, bool CLAIM = false, bool PEER = false>
+//
+// LINKED (the paper's single-scan partitioning, P593-597: "we scan the data
+// once and write them to a linked list of buffers managed with atomic
+// operations"): no histogram precedes the pass.  offsets[b] = lk.cnt[b] is
+// the bucket's running tuple count; a claimed run [pos, pos + c) of bucket b
+// lives in buffers pos / buf .. (pos + c - 1) / buf of b's chain.  The
+// claimant of a run that contains a buffer's first position allocates that
+// buffer (one atomic on the pool), publishes it in the directory, and only
+// then waits for the buffer its own run starts in, which the earlier
+// claimant of that buffer's first position allocates without waiting on
+// anything -- so every wait ends.  A run (<= one tile <= buf tuples) spans at
+// most two buffers.
+template <int KW, int PW, bool AOS, class C, bool IDENT, bool CLAIM = false, bool PEER = false,
+          bool LINKED = false>
 __global__ void __launch_bounds__(C::NT, C::MINB)
 k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ offsets,
           Tup<KW, PW>* __restrict__ out, Tup<KW, PW>* const* __restrict__ peer_out = nullptr,
-          uint32_t agg = 0) {
+          uint32_t agg = 0, LinkMap lk = LinkMap{}) {
   static_assert(!PEER || CLAIM, "peer scatters claim their runs");
+  static_assert(!LINKED || (CLAIM && !PEER), "linked scatters claim their runs into local chains");
   using K = typename UW<KW>::T;
   using V = typename UW<PW>::T;
   using Tp = Tup<KW, PW>;
@@ -682,6 +734,8 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
   uint32_t* s_wt = s_cur + P4;                        // warp totals
   uint64_t* bar = reinterpret_cast<uint64_t*>(s_wt + 64);
   Tup<KW, PW>** s_out = reinterpret_cast<Tup<KW, PW>**>(bar + STAGES + 8);  // PEER: [P] destinations
+  uint32_t* s_sp = reinterpret_cast<uint32_t*>(bar + STAGES + 8);   // LINKED: [P] tile position of the buffer switch
+  uint32_t* s_dl2 = s_sp + P4;                                      // LINKED: [P] second buffer's run start - tile start
 
   uint32_t seg, j, lo, hi;
   if constexpr (CLAIM) seg_chunk_tiles(m, blockIdx.x, (uint32_t)C::T, seg, j, lo, hi);
@@ -815,6 +869,31 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
         }
           s_st[b] = ex;
           s_dl[b] = run - ex;
+          if constexpr (LINKED) {
+            if (c) {
+              const uint32_t B = lk.buf;
+              const uint32_t k0 = run / B, k1 = (run + c - 1) / B;
+              uint32_t* drow = lk.dir + (size_t)b * lk.kmax;
+              // the buffers whose first position lies in this run are ours to allocate
+              for (uint32_t k = k0; k <= k1; k++) {
+                if (k * B < run) continue;
+                const uint32_t id = atomicAdd(lk.pool, 1u);
+                lk.owner[id] = b;
+                lk.kidx[id] = k;
+                __threadfence();
+                atomicExch(drow + k, id + 1u);
+              }
+              auto wait_id = [&](uint32_t k) -> uint32_t {
+                uint32_t v;
+                while ((v = *reinterpret_cast<volatile uint32_t*>(drow + k)) == 0u) __nanosleep(64);
+                return v - 1u;
+              };
+              const uint32_t id0 = wait_id(k0), id1 = k1 != k0 ? wait_id(k1) : id0;
+              s_dl[b] = id0 * B - k0 * B + run - ex;
+              s_sp[b] = (k0 + 1) * B - run + ex;
+              s_dl2[b] = id1 * B - k1 * B + run - ex;
+            }
+          }
           s_cnt[b] = 0;
           ex += c;
         }
@@ -854,7 +933,10 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
     // random shared-memory store + load)
     auto dst_of = [&](uint32_t i, const Tp& y) -> uint32_t {
       if constexpr (C::DST) return s_dst[i];
-      else return s_dl[bucket_of(part_hash<KW, IDENT>(y.k), bf)] + i;
+      else if constexpr (LINKED) {
+        const uint32_t b = bucket_of(part_hash<KW, IDENT>(y.k), bf);
+        return (i < s_sp[b] ? s_dl[b] : s_dl2[b]) + i;
+      } else return s_dl[bucket_of(part_hash<KW, IDENT>(y.k), bf)] + i;
     };
     if constexpr (PEER) {
       auto put = [&](uint32_t i) {

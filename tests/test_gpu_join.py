@@ -474,3 +474,47 @@ print("ok")
     env = dict(os.environ, HAPE_JOINT="0", PYTHONPATH=root)
     r = subprocess.run([sys.executable, "-c", code], cwd=root, env=env, capture_output=True, text=True, timeout=600)
     assert r.returncode == 0 and "ok" in r.stdout, r.stdout + r.stderr
+
+
+# ---- the paper's single-scan linked-buffer pass 1 (HAPE_FLAG_LINKED, NEXT-2) --
+@pytest.mark.parametrize("bits", [(8, 8), (3, 5), (10, 10), (12, 4), (6, 12)])
+@pytest.mark.parametrize("cfg", ["c2", "c3", "dup", "c5"])
+def test_linked_pass1_vs_oracle(cfg, bits):
+    n = {"c2": 1 << 20, "c3": 1 << 18, "dup": 20000, "c5": 1 << 19}[cfg]
+    kw = dict(dup_domain=300) if cfg == "dup" else (dict(theta=1.0) if cfg == "c5" else {})
+    wl = datagen.make(cfg, n_r=n, n_s=2 * n + 77, **kw)
+    kdt = DT[wl.key_bits]
+    want = oracle_res(wl.R.key, wl.R.payload, wl.S.key, wl.S.payload, materialize=cfg != "c5")
+    j = joiner(kdt, radix_passes=2, radix_bits=bits, linked=True)
+    out = None
+    if cfg != "c5":
+        out = (torch.empty(max(want["count"], 1), dtype=kdt, device="cuda"),
+               torch.empty(max(want["count"], 1), dtype=kdt, device="cuda"))
+    res = j.join(cuda(wl.R.key), cuda(wl.R.payload), cuda(wl.S.key), cuda(wl.S.payload), *(out or (None, None)))
+    check(res, want)
+    if out is not None:
+        a, b = sorted_pairs(out[0][:want["count"]], out[1][:want["count"]])
+        assert np.array_equal(a, want["pairs"][0]) and np.array_equal(b, want["pairs"][1])
+    # repeated call (graph replay, directory reset inside the graph)
+    res2 = j.join(cuda(wl.R.key), cuda(wl.R.payload), cuda(wl.S.key), cuda(wl.S.payload), *(out or (None, None)))
+    assert res2.as_tuple() == res.as_tuple()
+
+
+@pytest.mark.parametrize("bits,kb", [((8, 8), 32), ((5, 7), 64), ((11, 9), 32)])
+def test_linked_partition_invariants(bits, kb):
+    n = (1 << 20) + 777
+    rng = np.random.default_rng(13)
+    kdt = np.int32 if kb == 32 else np.int64
+    keys = rng.integers(np.iinfo(kdt).min, np.iinfo(kdt).max, n, dtype=kdt)
+    keys[: n // 5] = keys[0]                      # a hot key: one chain far longer than the others
+    pays = np.arange(n).astype(kdt)
+    j = joiner(DT[kb], radix_passes=2, radix_bits=bits, linked=True)
+    ok, op, ob, plan = j.debug_partition(cuda(keys), cuda(pays))
+    ok, op, ob = ok.cpu().numpy(), op.cpu().numpy(), ob.cpu().numpy()
+    b1, b2 = bits
+    Q = 1 << (b1 + b2)
+    assert ob[0] == 0 and ob[-1] == n and np.all(np.diff(ob) >= 0) and len(ob) == Q + 1
+    assert np.array_equal(np.sort(op), pays)
+    assert np.array_equal(ok, keys[op.astype(np.int64)])
+    pid = partition.partition_id(ok, b1, b2)
+    assert np.array_equal(pid, np.repeat(np.arange(Q), np.diff(ob)))
