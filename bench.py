@@ -276,7 +276,8 @@ def time_calls(fn, steps, stream):
     return e0.elapsed_time(e1) / steps, {k: v / steps for k, v in stage_sum.items()}, launches, res
 
 
-def run_leg(name, cfg, args, peak, n_r=None, n_s=None, theta=1.0, r_unique=True, materialize=None, steps=None):
+def run_leg(name, cfg, args, peak, n_r=None, n_s=None, theta=1.0, r_unique=True, materialize=None, steps=None,
+            linked=False):
     """One extra single-GPU workload (a bench 'leg'): generate, warm up, time."""
     import torch
     import datagen
@@ -293,7 +294,7 @@ def run_leg(name, cfg, args, peak, n_r=None, n_s=None, theta=1.0, r_unique=True,
         out_r = torch.empty(n_s, dtype=rp.dtype, device="cuda")
         out_s = torch.empty(n_s, dtype=sp.dtype, device="cuda")
     j = RadixJoin(key_dtype=rk.dtype, r_payload_dtype=rp.dtype, s_payload_dtype=sp.dtype,
-                  max_r=n_r, max_s=n_s, r_unique=r_unique, stream=torch.cuda.current_stream())
+                  max_r=n_r, max_s=n_s, r_unique=r_unique, linked=linked, stream=torch.cuda.current_stream())
     for _ in range(args.warmup):
         res = j.join(rk, rp, sk, sp, out_r, out_s)
     torch.cuda.synchronize()
@@ -302,7 +303,8 @@ def run_leg(name, cfg, args, peak, n_r=None, n_s=None, theta=1.0, r_unique=True,
     kw, prw, psw = rk.element_size(), rp.element_size(), sp.element_size()
     roof = roofline_of(res, st, ms, kw, prw, psw, mat, peak)
     leg = {"workload": f"{cfg}: {CONFIG_TEXT.get(cfg, cfg)}" + (f"; theta={theta}" if cfg == "c5" else "")
-           + ("" if r_unique else "; bag-semantics probe (R not declared unique)"),
+           + ("" if r_unique else "; bag-semantics probe (R not declared unique)")
+           + ("; pass 1 = single-scan linked-buffer partitioning (P593-597)" if linked else ""),
            "n_r": n_r, "n_s": n_s, "steps": k, "ms_per_step": round(ms, 4), "value": (n_r + n_s) / (ms / 1000.0),
            "unit": UNIT, "passes": res.passes, "bits": list(res.bits), "n_items": res.n_items,
            "match_count": res.match_count, "r_unique_declared": r_unique, "materialize": mat,
@@ -341,6 +343,9 @@ def main():
                     help="extra single-GPU workloads at N=1, comma list of c1,c3,c4,c2bag,c5 (or c5:THETA); "
                          "'default' = c1,c3,c4,c2bag,c5:0.5,c5:0.75,c5:0.9,c5:1.0; 'none'")
     ap.add_argument("--leg-steps", type=int, default=5)
+    ap.add_argument("--partitioner", default="hist", choices=["hist", "linked"],
+                    help="pass 1: histogram -> prefix sum -> scatter (default), or the paper's single-scan "
+                         "linked-buffer partitioning (HAPE_FLAG_LINKED; A/B, SURVEY NEXT-2)")
     ap.add_argument("--no-ablation", action="store_true",
                     help="skip the non-partitioned GPU join comparison (PAPER.md Fig. 6)")
     ap.add_argument("--no-coprocess", action="store_true",
@@ -395,7 +400,7 @@ def main():
     j = RadixJoin(key_dtype=kdt, r_payload_dtype=pdt, s_payload_dtype=pdt, device=local,
                   max_r=nr_loc, max_s=ns_loc, world_size=world, rank=rank,
                   radix_passes=args.passes, radix_bits=tuple(int(x) for x in args.bits.split(",")),
-                  r_unique=not args.bag, nccl_comm=comm, stream=stream)
+                  r_unique=not args.bag, nccl_comm=comm, stream=stream, linked=args.partitioner == "linked")
     assert j.stream.cuda_stream == stream.cuda_stream
     out_r = out_s = None
     if materialize:
@@ -581,11 +586,14 @@ def main():
     # ---- the other BASELINE configs on this one GPU (extra keys of the line)
     legs = {}
     if world == 1 and args.legs != "none":
-        spec = args.legs if args.legs != "default" else "c1,c3,c4,c2bag,c5:0.5,c5:0.75,c5:0.9,c5:1.0"
+        spec = args.legs if args.legs != "default" else \
+            "c1,c3,c4,c2bag,c2linked,c4linked,c5:0.5,c5:0.75,c5:0.9,c5:1.0"
         for item in [x for x in spec.split(",") if x]:
             try:
                 if item == "c2bag":
                     legs[item] = run_leg(item, "c2", args, peak, r_unique=False)
+                elif item in ("c2linked", "c4linked"):
+                    legs[item] = run_leg(item, item[:2], args, peak, linked=True)
                 elif item.startswith("c5"):
                     th = float(item.split(":")[1]) if ":" in item else 1.0
                     legs[f"c5_theta{th}"] = run_leg(item, "c5", args, peak, theta=th)
@@ -619,6 +627,7 @@ def main():
                        "n_r": n_r, "n_s": n_s, "per_rank_r": nr_loc, "per_rank_s": ns_loc,
                        "passes": res.passes, "bits": list(res.bits), "n_items": res.n_items,
                        "r_unique_declared": not args.bag,
+                       "partitioner": args.partitioner,
                        "materialize": materialize,
                        "l2": "inputs and workspace (>=2 GiB per step) exceed the 126 MB L2; no flush needed",
                        "parallelism": f"hash-sharded x{world}" if world > 1 else "1 GPU"},
