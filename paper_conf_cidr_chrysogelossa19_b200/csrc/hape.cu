@@ -452,6 +452,10 @@ static hape_status launch_scatter_linked(hape_join* h, int kw, const Src& s, Seg
 static uint32_t lb_buf(size_t tb) { return tb <= 8 ? 2u * 512u * 13u : 2u * 384u * 9u; }
 static uint64_t lb_nbuf(uint64_t n, size_t tb, uint32_t P1) { return (n + lb_buf(tb) - 1) / lb_buf(tb) + P1; }
 static uint64_t lb_kmax(uint64_t n, size_t tb) { return (n + lb_buf(tb) - 1) / lb_buf(tb) + 1; }
+// linked pass 1: directory [P1][kmax] + owner [nbuf] + chain index [nbuf]
+static size_t lb_ws_bytes(uint64_t n, size_t tb, uint32_t P1) {
+  return (size_t)P1 * lb_kmax(n, tb) * 4 + 2 * lb_nbuf(n, tb, P1) * 4 + 64;
+}
 
 // scatter shape per tuple width (measured best of the ScCfg sweep);
 // (the destination-table variant ScCfg<..., DST=true> is no longer dispatched)
@@ -468,6 +472,11 @@ static hape_status scatter_i(hape_join* h, const Src& s, SegMap m, BitField bf, 
   if constexpr (KW + PW <= 8) {
     if (v == 1) return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
     if (v == 2) return scatter_t<KW, PW, AOS, ScCfg<512, 12, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
+    // wide fan-outs (>= 1024 buckets): one CTA per SM staging twice the tile
+    // (longer runs per bucket and tile); HAPE_SC=3 forces it, HAPE_SC_WIDE=1 for P >= 1024
+    static int wide = [] { const char* e = getenv("HAPE_SC_WIDE"); return e ? atoi(e) : 0; }();
+    if (v == 3 || (wide && P >= 1024))
+      return scatter_t<KW, PW, AOS, ScCfg<1024, 12, 2, 1>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
     return scatter_t<KW, PW, AOS, ScCfg<512, 13, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
   } else {
     static int w = [] { const char* e = getenv("HAPE_SC16"); return e ? atoi(e) : 0; }();
@@ -873,8 +882,8 @@ static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const
       const size_t tb = tup_bytes(kw, io[s].in.pw);
       const uint32_t B = lb_buf(tb);
       const uint64_t nb = lb_nbuf(n, tb, P1), km = lb_kmax(n, tb);
-      const size_t dir_b = (size_t)P1 * km * 4;
-      CKS(ensure(h, h->lbuf[s], dir_b + 2 * nb * 4 + 64));
+      if (h->lbuf[s].bytes < lb_ws_bytes(n, tb, P1))
+        return fail(h, HAPE_ERR_INVALID_ARG, "linked-buffer workspace not allocated before the passes");
       uint32_t* dir = static_cast<uint32_t*>(h->lbuf[s].p);
       uint32_t* owner = dir + (size_t)P1 * km;
       uint32_t* kidx = owner + nb;
@@ -1237,6 +1246,15 @@ static void stage_times(hape_join* h, hape_join_result* res) {
   (void)cudaGetLastError();
 }
 
+
+// allocations of the passes that must precede enqueueing (CUDA-graph capture)
+static hape_status ensure_pass_ws(hape_join* h, const hape_plan& pl, const uint64_t* n, const int* pw, int nside) {
+  if (!use_linked(h, pl)) return HAPE_OK;
+  const int kw = key_width(h->cfg);
+  for (int s = 0; s < nside; s++) CKS(ensure(h, h->lbuf[s], lb_ws_bytes(n[s], tup_bytes(kw, pw[s]), 1u << pl.bits[0])));
+  return HAPE_OK;
+}
+
 // pass-1 output bytes: the relation, or (linked pass 1) its buffer pool
 static size_t ping_bytes(const hape_join* h, const hape_plan& pl, uint64_t n, size_t tb) {
   if (use_linked(h, pl)) return (size_t)lb_nbuf(n, tb, 1u << pl.bits[0]) * lb_buf(tb) * tb + 16;
@@ -1273,6 +1291,7 @@ static hape_status local_join(hape_join* h, const Src loc_in[2], const MatOut& m
     CKS(ensure(h, h->ping[s], ping_bytes(h, pl, n_loc[s], tup_bytes(kw, pw[s]))));
     if (pl.passes == 2) CKS(ensure(h, h->pong[s], n_loc[s] * tup_bytes(kw, pw[s]) + 16));
   }
+  CKS(ensure_pass_ws(h, pl, n_loc, pw, 2));
   const uint32_t Q = 1u << (pl.bits[0] + (pl.passes == 2 ? pl.bits[1] : 0));
   uint32_t* ctrs = at<uint32_t>(h, L.ctrs);  // [0] n_items
   auto enqueue = [&]() -> hape_status {
@@ -1987,6 +2006,11 @@ hape_status hape_debug_partition(hape_join* h, const hape_relation* rel, int is_
   CKS(ensure(h, h->small, L.total));
   CKS(ensure(h, h->ping[0], ping_bytes(h, pl, rel->n, tup_bytes(kw, pw))));
   CKS(ensure(h, h->pong[0], rel->n * tup_bytes(kw, pw) + 16));
+  {
+    const uint64_t nn[1] = {rel->n};
+    const int pp[1] = {pw};
+    CKS(ensure_pass_ws(h, pl, nn, pp, 1));
+  }
   CK(h, cudaMemsetAsync(at<char>(h, L.zero_lo), 0, L.zero_hi - L.zero_lo, h->stream));
   PassIO io[2];
   io[0] = PassIO{in, h->ping[0].p, h->pong[0].p};
