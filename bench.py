@@ -230,14 +230,17 @@ KERNEL_NAME = {"hist1": "k_hist pass 1 (R+S)", "scatter1": "k_scatter pass 1 (R+
                "build_probe": "k_build_probe", "devpart": "device partition (hist+scan+scatter)"}
 
 
-def is_joint(res):
-    return (res.passes == 2 and 6 <= res.bits[0] + res.bits[1] <= 16
+def is_joint(res, linked=False):
+    return (not linked and res.passes == 2 and 6 <= res.bits[0] + res.bits[1] <= 16
             and os.environ.get("HAPE_JOINT", "1") != "0")
 
 
-def roofline_of(res, stage_avg, ms, kw, prw, psw, materialize, peak, extra=None):
-    joint = is_joint(res)
+def roofline_of(res, stage_avg, ms, kw, prw, psw, materialize, peak, extra=None, linked=False):
+    joint = is_joint(res, linked)
     alg = alg_bytes(res, kw, prw, psw, materialize, joint)
+    if linked:
+        # pass 1 without a histogram: stage hist1 is the buffer-directory reset
+        alg.pop("hist1", None)
     alg.update(extra or {})
     per_stage = {}
     for k in alg:
@@ -301,7 +304,7 @@ def run_leg(name, cfg, args, peak, n_r=None, n_s=None, theta=1.0, r_unique=True,
     k = steps or args.leg_steps
     ms, st, launches, res = time_calls(lambda: j.join(rk, rp, sk, sp, out_r, out_s), k, j.stream)
     kw, prw, psw = rk.element_size(), rp.element_size(), sp.element_size()
-    roof = roofline_of(res, st, ms, kw, prw, psw, mat, peak)
+    roof = roofline_of(res, st, ms, kw, prw, psw, mat, peak, linked=linked)
     leg = {"workload": f"{cfg}: {CONFIG_TEXT.get(cfg, cfg)}" + (f"; theta={theta}" if cfg == "c5" else "")
            + ("" if r_unique else "; bag-semantics probe (R not declared unique)")
            + ("; pass 1 = single-scan linked-buffer partitioning (P593-597)" if linked else ""),
@@ -452,7 +455,8 @@ def main():
         # NCCL form: destination hist + scatter into a send buffer; fused form:
         # the destination totals only (the scatter is the exchange stage)
         extra["devpart"] = (kw if fused else kw + 2 * t) * (nr_loc + ns_loc)
-    roofline = roofline_of(res, stage_avg, ms, kw, pw, pw, materialize, peak, extra)
+    roofline = roofline_of(res, stage_avg, ms, kw, pw, pw, materialize, peak, extra,
+                           linked=args.partitioner == "linked")
     roofline["peak_source"] = peak_src
     traffic = None
     try:

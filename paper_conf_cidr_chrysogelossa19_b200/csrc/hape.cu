@@ -447,9 +447,11 @@ static hape_status launch_scatter_linked(hape_join* h, int kw, const Src& s, Seg
 #undef HAPE_SCL
 }
 
-// linked-buffer geometry: buffers of two default scatter tiles (pass 2 reads
-// whole tiles), a dense directory row of kmax entries per pass-1 bucket
-static uint32_t lb_buf(size_t tb) { return tb <= 8 ? 2u * 512u * 13u : 2u * 384u * 9u; }
+// linked-buffer geometry: buffers of eight default scatter tiles (pass 2
+// reads whole tiles, one CTA per buffer: 2-tile buffers measured 48.5 vs
+// 23.3 ms for C4's pass 2 -- per-CTA set-up), a dense directory row of kmax
+// entries per pass-1 bucket
+static uint32_t lb_buf(size_t tb) { return tb <= 8 ? 8u * 512u * 13u : 8u * 384u * 9u; }
 static uint64_t lb_nbuf(uint64_t n, size_t tb, uint32_t P1) { return (n + lb_buf(tb) - 1) / lb_buf(tb) + P1; }
 static uint64_t lb_kmax(uint64_t n, size_t tb) { return (n + lb_buf(tb) - 1) / lb_buf(tb) + 1; }
 // linked pass 1: directory [P1][kmax] + owner [nbuf] + chain index [nbuf]
@@ -473,10 +475,12 @@ static hape_status scatter_i(hape_join* h, const Src& s, SegMap m, BitField bf, 
     if (v == 1) return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
     if (v == 2) return scatter_t<KW, PW, AOS, ScCfg<512, 12, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
     // wide fan-outs (>= 1024 buckets): one CTA per SM staging twice the tile
-    // (longer runs per bucket and tile); HAPE_SC=3 forces it, HAPE_SC_WIDE=1 for P >= 1024
-    static int wide = [] { const char* e = getenv("HAPE_SC_WIDE"); return e ? atoi(e) : 0; }();
-    if (v == 3 || (wide && P >= 1024))
-      return scatter_t<KW, PW, AOS, ScCfg<1024, 12, 2, 1>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
+    // (longer runs per bucket and tile); HAPE_SC=3 forces it, used for P >= 1024 unless HAPE_SC_WIDE=0
+    // (measured C4 at N=1, 2 x 1024 buckets: scatters 25.0 / 23.3 -> 18.8 / 18.4 ms)
+    static int wide = [] { const char* e = getenv("HAPE_SC_WIDE"); return e ? atoi(e) : 1; }();
+    using Cw = ScCfg<1024, 12, 2, 1>;
+    if (v == 3 || (wide && P >= 1024 && ScLayout<KW, PW, AOS, Cw>::bytes(P) <= 220 * 1024))
+      return scatter_t<KW, PW, AOS, Cw, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
     return scatter_t<KW, PW, AOS, ScCfg<512, 13, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
   } else {
     static int w = [] { const char* e = getenv("HAPE_SC16"); return e ? atoi(e) : 0; }();

@@ -658,7 +658,7 @@ struct ScLayout {
   static __host__ __device__ constexpr size_t bytes(uint32_t P, bool peer = false, bool linked = false) {
     return C::STAGES * RAW + (C::DST ? (size_t)T * 4 : 0) + (size_t)((P + 3) & ~3u) * 16 + 64 * 4 +
            C::STAGES * 8 + 64 + (peer ? (size_t)((P + 1) & ~1u) * 8 : 0) +
-           (linked ? (size_t)((P + 3) & ~3u) * 8 : 0);
+           (linked ? (size_t)((P + 3) & ~3u) * 12 : 0);
   }
 };
 
@@ -734,8 +734,8 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
   uint32_t* s_wt = s_cur + P4;                        // warp totals
   uint64_t* bar = reinterpret_cast<uint64_t*>(s_wt + 64);
   Tup<KW, PW>** s_out = reinterpret_cast<Tup<KW, PW>**>(bar + STAGES + 8);  // PEER: [P] destinations
-  uint32_t* s_sp = reinterpret_cast<uint32_t*>(bar + STAGES + 8);   // LINKED: [P] tile position of the buffer switch
-  uint32_t* s_dl2 = s_sp + P4;                                      // LINKED: [P] second buffer's run start - tile start
+  uint2* s_dlsp = reinterpret_cast<uint2*>(bar + STAGES + 8);      // LINKED: [P] {run start - tile start, buffer switch}
+  uint32_t* s_dl2 = reinterpret_cast<uint32_t*>(s_dlsp + P4);       // LINKED: [P] second buffer's run start - tile start
 
   uint32_t seg, j, lo, hi;
   if constexpr (CLAIM) seg_chunk_tiles(m, blockIdx.x, (uint32_t)C::T, seg, j, lo, hi);
@@ -889,8 +889,7 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
                 return v - 1u;
               };
               const uint32_t id0 = wait_id(k0), id1 = k1 != k0 ? wait_id(k1) : id0;
-              s_dl[b] = id0 * B - k0 * B + run - ex;
-              s_sp[b] = (k0 + 1) * B - run + ex;
+              s_dlsp[b] = make_uint2(id0 * B - k0 * B + run - ex, (k0 + 1) * B - run + ex);
               s_dl2[b] = id1 * B - k1 * B + run - ex;
             }
           }
@@ -934,8 +933,11 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
     auto dst_of = [&](uint32_t i, const Tp& y) -> uint32_t {
       if constexpr (C::DST) return s_dst[i];
       else if constexpr (LINKED) {
+        // one 8-byte load; the second buffer's start only for the rare
+        // tuples past a buffer boundary
         const uint32_t b = bucket_of(part_hash<KW, IDENT>(y.k), bf);
-        return (i < s_sp[b] ? s_dl[b] : s_dl2[b]) + i;
+        const uint2 v = s_dlsp[b];
+        return (i < v.y ? v.x : s_dl2[b]) + i;
       } else return s_dl[bucket_of(part_hash<KW, IDENT>(y.k), bf)] + i;
     };
     if constexpr (PEER) {
