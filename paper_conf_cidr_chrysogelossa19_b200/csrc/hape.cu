@@ -406,13 +406,16 @@ static hape_status launch_scan(hape_join* h, SegMap m, uint32_t P, uint32_t* his
   return HAPE_OK;
 }
 
+// dynamic shared memory a scatter CTA may opt into (B200: 227 KB per block)
+constexpr size_t kScatterSmemMax = 232448 - 1024;
+
 template <int KW, int PW, bool AOS, class C, bool IDENT, bool CLAIM, bool LINKED = false>
 static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* offs,
                              void* out, const LinkMap* lk = nullptr) {
   const size_t smem = ScLayout<KW, PW, AOS, C>::bytes(P, false, LINKED);
   static uint64_t attr_dev = 0;
   auto kern = k_scatter<KW, PW, AOS, C, IDENT, CLAIM, false, LINKED>;
-  CKS(smem_attr(h, kern, 220 * 1024, attr_dev));
+  CKS(smem_attr(h, kern, (int)kScatterSmemMax, attr_dev));
   const unsigned grid = m.nseg * m.cps;
   if (grid == 0) return HAPE_OK;
   // warp-aggregated ranking: always for narrow fan-outs (the destination
@@ -425,14 +428,28 @@ static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, 
   return HAPE_OK;
 }
 
-// pass 1 of the linked-buffer partitioning (k_scatter LINKED), default shapes
-template <int KW, int PW, bool AOS>
-static hape_status scatter_linked_v(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, void* out,
+// pass 1 of the linked-buffer partitioning (k_scatter LINKED): the shape
+// the hist path would use where it fits with the chain arrays (wide tiles
+// for >= 1024 buckets), else a smaller tile (runs <= one tile <= a buffer)
+template <int KW, int PW, bool AOS, class C>
+static hape_status scatter_linked_c(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, void* out,
                                     const LinkMap& lk) {
-  using C = typename std::conditional<KW + PW <= 8, ScCfg<512, 13, 2, 2>, ScCfg<384, 9, 2, 2>>::type;
   if (h->cfg.part_fn == HAPE_PART_IDENTITY)
     return scatter_t<KW, PW, AOS, C, true, true, true>(h, s, m, bf, P, lk.cnt, out, &lk);
   return scatter_t<KW, PW, AOS, C, false, true, true>(h, s, m, bf, P, lk.cnt, out, &lk);
+}
+
+template <int KW, int PW, bool AOS>
+static hape_status scatter_linked_v(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, void* out,
+                                    const LinkMap& lk) {
+  using Cd = typename std::conditional<KW + PW <= 8, ScCfg<512, 13, 2, 2>, ScCfg<384, 9, 2, 2>>::type;
+  using Cw = ScCfg<1024, 12, 2, 1>;
+  using Cs = ScCfg<256, 8, 2, 1>;
+  if (KW + PW <= 8 && P >= 1024 && ScLayout<KW, PW, AOS, Cw>::bytes(P, false, true) <= kScatterSmemMax)
+    return scatter_linked_c<KW, PW, AOS, Cw>(h, s, m, bf, P, out, lk);
+  if (ScLayout<KW, PW, AOS, Cd>::bytes(P, false, true) <= kScatterSmemMax)
+    return scatter_linked_c<KW, PW, AOS, Cd>(h, s, m, bf, P, out, lk);
+  return scatter_linked_c<KW, PW, AOS, Cs>(h, s, m, bf, P, out, lk);
 }
 
 static hape_status launch_scatter_linked(hape_join* h, int kw, const Src& s, SegMap m, BitField bf, uint32_t P,
@@ -479,7 +496,7 @@ static hape_status scatter_i(hape_join* h, const Src& s, SegMap m, BitField bf, 
     // (measured C4 at N=1, 2 x 1024 buckets: scatters 25.0 / 23.3 -> 18.8 / 18.4 ms)
     static int wide = [] { const char* e = getenv("HAPE_SC_WIDE"); return e ? atoi(e) : 1; }();
     using Cw = ScCfg<1024, 12, 2, 1>;
-    if (v == 3 || (wide && P >= 1024 && ScLayout<KW, PW, AOS, Cw>::bytes(P) <= 220 * 1024))
+    if (v == 3 || (wide && P >= 1024 && ScLayout<KW, PW, AOS, Cw>::bytes(P) <= kScatterSmemMax))
       return scatter_t<KW, PW, AOS, Cw, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
     return scatter_t<KW, PW, AOS, ScCfg<512, 13, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
   } else {
