@@ -334,7 +334,17 @@ static uint32_t joint_grid(const hape_join* h, uint32_t nchunks) {
   return std::max<uint32_t>(1, std::min<uint32_t>((uint32_t)h->num_sms, nchunks));
 }
 
-static size_t joint_smem(uint32_t P1, uint32_t P2) { return (size_t)P1 * P2 * 2 + (size_t)P1 * 4; }
+static size_t joint_smem(uint32_t P1, uint32_t P2, bool tma = false) {
+  if (!tma) return (size_t)P1 * P2 * 2 + (size_t)P1 * 4;
+  return hj_ring_off(P1 * P2 / 2, P1) + (size_t)HJ_NS * HJ_SB + 2 * HJ_NS * 8 + HJ_NS * 4 + 64;
+}
+
+// TMA-fed joint histogram where the ring fits beside the counters
+// (HAPE_HJ_TMA=0 keeps the register-batched loads)
+static bool hj_tma(uint32_t P1, uint32_t P2) {
+  static const int env = env_int("HAPE_HJ_TMA", 1);
+  return env != 0 && joint_smem(P1, P2, true) <= 200 * 1024;
+}
 
 // cudaFuncSetAttribute applies to the current device only: one bit per
 // device ordinal and kernel instantiation (the caller's `mask` is a static
@@ -351,10 +361,18 @@ static hape_status smem_attr(hape_join* h, F kern, int bytes, uint64_t& mask) {
 template <int KW, int PW, bool AOS, bool IDENT>
 static hape_status hist_joint_t(hape_join* h, const Src& s, SegMap m, BitField bf1, BitField bf2, uint32_t P1,
                                 uint32_t P2, uint32_t* rowsum, uint16_t* part, uint32_t* ovf) {
+  const uint32_t nch = m.nseg * m.cps;
+  if (hj_tma(P1, P2)) {
+    auto kern = k_hist_joint<KW, PW, AOS, IDENT, true>;
+    static uint64_t attr_dev = 0;
+    CKS(smem_attr(h, kern, 200 * 1024, attr_dev));
+    kern<<<joint_grid(h, nch), HJ_THREADS, joint_smem(P1, P2, true), h->stream>>>(s.in, m, P1, P2, rowsum, part,
+                                                                                ovf);
+    return HAPE_OK;
+  }
   auto kern = k_hist_joint<KW, PW, AOS, IDENT>;
   static uint64_t attr_dev = 0;
   CKS(smem_attr(h, kern, 200 * 1024, attr_dev));
-  const uint32_t nch = m.nseg * m.cps;
   kern<<<joint_grid(h, nch), HJ_THREADS, joint_smem(P1, P2), h->stream>>>(s.in, m, P1, P2, rowsum, part,
                                                                         ovf);
   return HAPE_OK;

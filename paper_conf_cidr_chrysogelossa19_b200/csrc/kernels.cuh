@@ -412,8 +412,18 @@ k_hist(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ hist
 // atomic per key.
 // --------------------------------------------------------------------------
 constexpr int HJ_THREADS = 1024;
+// TMA form: the keys stream through a ring of HJ_NS stages of HJ_SB bytes,
+// filled by the last warp with the bulk-copy engine (mbarrier full / empty
+// pairs) while 31 warps count -- bytes in flight without registers
+constexpr uint32_t HJ_SB = 16384;
+constexpr int HJ_NS = 4;
+constexpr int HJ_NCW = HJ_THREADS / 32 - 1;  // consumer warps
 
-template <int KW, int PW, bool AOS, bool IDENT>
+__host__ __device__ constexpr size_t hj_ring_off(uint32_t QW, uint32_t P1) {
+  return ((size_t)(QW + P1) * 4 + 127) / 128 * 128;
+}
+
+template <int KW, int PW, bool AOS, bool IDENT, bool TMA = false>
 __global__ void __launch_bounds__(HJ_THREADS, 1)
 k_hist_joint(PartIn in, SegMap m, uint32_t P1, uint32_t P2, uint32_t* __restrict__ rowsum, uint16_t* __restrict__ part, uint32_t* __restrict__ ovf) {
   extern __shared__ __align__(16) uint32_t sh_hj[];
@@ -477,25 +487,87 @@ k_hist_joint(PartIn in, SegMap m, uint32_t P1, uint32_t P2, uint32_t* __restrict
     }
   };
   const uint32_t nchunks = m.nseg * m.cps;
-  for (uint32_t c = blockIdx.x; c < nchunks; c += gridDim.x) {
-    uint32_t seg, j, lo, hi;
+  auto chunk_of = [&](uint32_t c, uint32_t& lo, uint32_t& vlo, uint32_t& vhi, uint32_t& hi) {
+    uint32_t seg, j;
     seg_chunk(m, c, seg, j, lo, hi);
-    uint32_t vlo = lo;
+    vlo = lo;
     while (vlo < hi && (reinterpret_cast<uintptr_t>(base + vlo) & 15)) vlo++;
-    const uint32_t nvec = (hi - vlo) / PER;
-    const uint32_t vhi = vlo + nvec * PER;
-    for (uint32_t i = lo + threadIdx.x; i < vlo; i += HJ_THREADS) count(key_of(base[i]));
-    for (uint32_t i = vhi + threadIdx.x; i < hi; i += HJ_THREADS) count(key_of(base[i]));
-    const uint4* __restrict__ vk = reinterpret_cast<const uint4*>(base + vlo);
-    uint32_t v = threadIdx.x;
-    for (; v + (HIST_VEC - 1) * HJ_THREADS < nvec; v += HIST_VEC * HJ_THREADS) {
-      uint4 w[HIST_VEC];
+    vhi = vlo + (hi - vlo) / PER * PER;
+  };
+  if constexpr (!TMA) {
+    for (uint32_t c = blockIdx.x; c < nchunks; c += gridDim.x) {
+      uint32_t lo, vlo, vhi, hi;
+      chunk_of(c, lo, vlo, vhi, hi);
+      const uint32_t nvec = (vhi - vlo) / PER;
+      for (uint32_t i = lo + threadIdx.x; i < vlo; i += HJ_THREADS) count(key_of(base[i]));
+      for (uint32_t i = vhi + threadIdx.x; i < hi; i += HJ_THREADS) count(key_of(base[i]));
+      const uint4* __restrict__ vk = reinterpret_cast<const uint4*>(base + vlo);
+      uint32_t v = threadIdx.x;
+      for (; v + (HIST_VEC - 1) * HJ_THREADS < nvec; v += HIST_VEC * HJ_THREADS) {
+        uint4 w[HIST_VEC];
 #pragma unroll
-      for (int u = 0; u < HIST_VEC; u++) w[u] = __ldcs(vk + v + u * HJ_THREADS);
+        for (int u = 0; u < HIST_VEC; u++) w[u] = __ldcs(vk + v + u * HJ_THREADS);
 #pragma unroll
-      for (int u = 0; u < HIST_VEC; u++) count_vec(w[u]);
+        for (int u = 0; u < HIST_VEC; u++) count_vec(w[u]);
+      }
+      for (; v < nvec; v += HJ_THREADS) count_vec(__ldcs(vk + v));
     }
-    for (; v < nvec; v += HJ_THREADS) count_vec(__ldcs(vk + v));
+  } else {
+    unsigned char* ring = reinterpret_cast<unsigned char*>(sh_hj) + hj_ring_off(QW, P1);
+    uint64_t* full = reinterpret_cast<uint64_t*>(ring + HJ_NS * HJ_SB);
+    uint64_t* empty = full + HJ_NS;
+    uint32_t* s_len = reinterpret_cast<uint32_t*>(empty + HJ_NS);
+    if (threadIdx.x == 0) {
+      for (int i = 0; i < HJ_NS; i++) { mbar_init(&full[i], 1); mbar_init(&empty[i], HJ_NCW); }
+      asm volatile("fence.mbarrier_init.release.cluster;" ::: "memory");
+    }
+    __syncthreads();
+    const int warp = threadIdx.x >> 5, lane = threadIdx.x & 31;
+    if (warp == HJ_NCW) {
+      // producer: every chunk's vector-aligned middle, stage by stage
+      if (lane == 0) {
+        const uint64_t pol = policy_evict_first();
+        uint32_t seq = 0;
+        for (uint32_t c = blockIdx.x; c < nchunks; c += gridDim.x) {
+          uint32_t lo, vlo, vhi, hi;
+          chunk_of(c, lo, vlo, vhi, hi);
+          const char* src = reinterpret_cast<const char*>(base + vlo);
+          const size_t nb = (size_t)(vhi - vlo) * ES;
+          for (size_t off = 0; off < nb; off += HJ_SB, seq++) {
+            const uint32_t st = seq % HJ_NS, ph = (seq / HJ_NS) & 1;
+            mbar_wait_backoff(&empty[st], ph ^ 1);
+            const uint32_t len = (uint32_t)min((size_t)HJ_SB, nb - off);
+            s_len[st] = len;
+            mbar_expect_tx(&full[st], len);
+            bulk_g2s(ring + (size_t)st * HJ_SB, src + off, len, &full[st], pol);
+          }
+        }
+        const uint32_t st = seq % HJ_NS, ph = (seq / HJ_NS) & 1;
+        mbar_wait_backoff(&empty[st], ph ^ 1);
+        s_len[st] = 0;  // end of the stream
+        mbar_arrive(&full[st]);
+      }
+    } else {
+      // consumers: unaligned heads / tails straight from HBM, then the ring
+      constexpr uint32_t NCT = HJ_NCW * 32;
+      for (uint32_t c = blockIdx.x; c < nchunks; c += gridDim.x) {
+        uint32_t lo, vlo, vhi, hi;
+        chunk_of(c, lo, vlo, vhi, hi);
+        for (uint32_t i = lo + threadIdx.x; i < vlo; i += NCT) count(key_of(base[i]));
+        for (uint32_t i = vhi + threadIdx.x; i < hi; i += NCT) count(key_of(base[i]));
+      }
+      for (uint32_t seq = 0;; seq++) {
+        const uint32_t st = seq % HJ_NS, ph = (seq / HJ_NS) & 1;
+        mbar_wait(&full[st], ph);
+        const uint32_t len = s_len[st];
+        if (len == 0) break;
+        const uint4* vp = reinterpret_cast<const uint4*>(ring + (size_t)st * HJ_SB);
+        const uint32_t nv = len / 16;
+        for (uint32_t v = threadIdx.x; v < nv; v += NCT) count_vec(vp[v]);
+        __syncwarp();
+        if (lane == 0) mbar_arrive(&empty[st]);
+      }
+    }
   }
   __syncthreads();
   // row totals of the 16-bit counters: a warp covers 32 consecutive words;

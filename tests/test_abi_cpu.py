@@ -88,3 +88,27 @@ def test_exchange_plan_matches_definition(lib, G):
         assert ro == np.concatenate([[0], np.cumsum(counts[:, me])[:-1]]).tolist()
         assert rt == int(counts[:, me].sum())
     assert lib.hape_exchange_plan(G, G, counts.reshape(-1).tolist())[0] == lib.HAPE_ERR_INVALID_ARG
+
+
+@pytest.mark.parametrize("G", [1, 2, 3, 8, 64])
+def test_peer_plan_tiles_every_receive_buffer(lib, G):
+    """hape_peer_plan (the fused exchange's addressing): the G sources'
+    segments tile each destination's receive buffer [0, total) exactly, in
+    rank order, and the capacity is the largest receive total."""
+    rng = np.random.default_rng(100 + G)
+    counts = rng.integers(0, 1000, (G, G))
+    counts[0, :] = 0                                  # a rank that sends nothing
+    offs = []
+    for me in range(G):
+        st, wo, rt, cap = lib.hape_peer_plan(G, me, counts.reshape(-1).tolist())
+        assert st == lib.HAPE_OK
+        assert rt == int(counts[:, me].sum()) and cap == int(counts.sum(axis=0).max())
+        offs.append(wo)
+    for d in range(G):
+        cover = np.zeros(int(counts[:, d].sum()), np.int64)
+        for src in range(G):
+            o, c = offs[src][d], int(counts[src, d])
+            assert o == int(counts[:src, d].sum())
+            cover[o:o + c] += 1
+        assert (cover == 1).all()
+    assert lib.hape_peer_plan(G, G, counts.reshape(-1).tolist())[0] == lib.HAPE_ERR_INVALID_ARG
