@@ -418,6 +418,7 @@ def test_open_addressing_refill_cases(identity):
 
 
 @pytest.mark.parametrize("env", [dict(HAPE_JOINT="0"), dict(HAPE_JOINT="0", HAPE_CLAIM="0"),
+                                 dict(HAPE_HJ_TMA="1"), dict(HAPE_SC="3"), dict(HAPE_SC_WIDE="0"),
                                  dict(HAPE_JN_OA="1"), dict(HAPE_JN_OA="1", HAPE_OA_NTAB="1"),
                                  dict(HAPE_JN_OA="1", HAPE_OA_U="4"), dict(HAPE_JN_OA="1", HAPE_OA_U="1")])
 def test_alternative_kernel_forms_vs_oracle(env):
