@@ -41,7 +41,10 @@ constexpr uint32_t kTargetPerPartition = 2048;  // R tuples per co-partition (Fi
 constexpr uint32_t kMaxBitsPerPass = 12;
 constexpr uint32_t kMaxSinglePassBits = 10;
 constexpr uint32_t kChunk = 32768;              // tuples per partitioning CTA (upper bound)
-constexpr uint32_t kMinChunk = 1024;
+// a partitioning CTA gets at least one full scatter tile (8-byte tuples):
+// smaller chunks pay a partial tile and P total / claim atomics each
+// (HAPE_MIN_CHUNK: A/B)
+constexpr uint32_t kMinChunk = 6656;
 
 inline uint32_t ceil_log2_u64(uint64_t x) {
   uint32_t b = 0;
@@ -198,7 +201,8 @@ static uint32_t cps_for(const hape_join* h, uint64_t total, uint32_t nseg) {
   const uint64_t want_ctas = (uint64_t)h->num_sms * 8;
   if (c * nseg < want_ctas) {
     uint64_t c2 = (want_ctas + nseg - 1) / nseg;
-    uint64_t cmax = std::max<uint64_t>(1, (avg + kMinChunk - 1) / kMinChunk);
+    static const uint64_t minc = [] { const char* e = getenv("HAPE_MIN_CHUNK"); return e ? (uint64_t)atoll(e) : (uint64_t)kMinChunk; }();
+    uint64_t cmax = std::max<uint64_t>(1, (avg + minc - 1) / minc);
     c = std::max<uint64_t>(c, std::min(c2, cmax));
   }
   return (uint32_t)std::max<uint64_t>(1, std::min<uint64_t>(c, 1u << 20));
