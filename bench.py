@@ -343,8 +343,8 @@ def main():
                     help="do not declare R's keys unique (HAPE_FLAG_R_UNIQUE): full bag-semantics probe")
     ap.add_argument("--theta", type=float, default=1.0, help="c5 Zipf skew")
     ap.add_argument("--legs", default="default",
-                    help="extra single-GPU workloads at N=1, comma list of c1,c3,c4,c2bag,c5 (or c5:THETA); "
-                         "'default' = c1,c3,c4,c2bag,c5:0.5,c5:0.75,c5:0.9,c5:1.0; 'none'")
+                    help="extra single-GPU workloads at N=1, comma list of c1,c3,c4,c4rG (C4's per-rank "
+                         "share at G ranks),c2bag,c2linked,c4linked,c5 (or c5:THETA); 'default' = all; 'none'")
     ap.add_argument("--leg-steps", type=int, default=5)
     ap.add_argument("--partitioner", default="hist", choices=["hist", "linked"],
                     help="pass 1: histogram -> prefix sum -> scatter (default), or the paper's single-scan "
@@ -591,13 +591,18 @@ def main():
     legs = {}
     if world == 1 and args.legs != "none":
         spec = args.legs if args.legs != "default" else \
-            "c1,c3,c4,c2bag,c2linked,c4linked,c5:0.5,c5:0.75,c5:0.9,c5:1.0"
+            "c1,c3,c4,c4r2,c4r4,c4r8,c2bag,c2linked,c4linked,c5:0.5,c5:0.75,c5:0.9,c5:1.0"
         for item in [x for x in spec.split(",") if x]:
             try:
                 if item == "c2bag":
                     legs[item] = run_leg(item, "c2", args, peak, r_unique=False)
                 elif item in ("c2linked", "c4linked"):
                     legs[item] = run_leg(item, item[:2], args, peak, linked=True)
+                elif item.startswith("c4r"):
+                    # the local join one rank runs after the exchange at G = 2/4/8
+                    # (2^31 / G tuples of R and of S, the C4 recipe)
+                    g = int(item[3:])
+                    legs[item] = run_leg(item, "c4", args, peak, n_r=(1 << 31) // g, n_s=(1 << 31) // g)
                 elif item.startswith("c5"):
                     th = float(item.split(":")[1]) if ":" in item else 1.0
                     legs[f"c5_theta{th}"] = run_leg(item, "c5", args, peak, theta=th)

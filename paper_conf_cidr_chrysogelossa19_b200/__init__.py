@@ -176,9 +176,11 @@ class RadixJoin:
         dev = self.cfg.device
         cur = torch.cuda.current_stream(dev)
         if cur.cuda_stream != self._stream_handle:
-            ev = torch.cuda.Event()
-            ev.record(cur)
-            torch.cuda.ExternalStream(self._stream_handle, device=dev).wait_event(ev)
+            if getattr(self, "_ext", None) is None:
+                self._ext = torch.cuda.ExternalStream(self._stream_handle, device=dev)
+                self._ev = torch.cuda.Event()
+            self._ev.record(cur)
+            self._ext.wait_event(self._ev)
 
     @property
     def stream(self):

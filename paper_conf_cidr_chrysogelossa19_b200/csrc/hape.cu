@@ -1276,6 +1276,8 @@ static hape_status exchange_p2p(hape_join* h, Src in[2], Src out[2]) {
 // stage times after the final event: each used stage runs until the next
 // used stage mark (stages are marked in enum order on the join stream)
 static void stage_times(hape_join* h, hape_join_result* res) {
+  static const bool off = getenv("HAPE_NO_STAGE_TIMES") != nullptr;  // (host-overhead A/B only)
+  if (off) return;
   int order[HAPE_NSTAGES];
   int no = 0;
   for (int s = HAPE_STAGE_H2D; s < HAPE_STAGE_TOTAL; s++)
@@ -1505,6 +1507,10 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
     CKN(h, ncclAllReduce(acc, acc, 4, ncclUint64, ncclSum, h->comm, h->stream));
     CK(h, cudaMemcpyAsync(h->h_res + 6, acc, 4 * 8, cudaMemcpyDeviceToHost, h->stream));
   }
+  // without host-resident pairs to copy back, the end-of-call event goes in
+  // now and one synchronisation serves both the result and the stage times
+  const bool host_pairs = mat && out->mem == HAPE_MEM_HOST;
+  if (!host_pairs) cudaEventRecord(h->ev[HAPE_NSTAGES], h->stream);
   CK(h, cudaStreamSynchronize(h->stream));
   const unsigned long long* r = h->h_res;
   res->local_match_count = r[0];
@@ -1521,12 +1527,14 @@ static hape_status join_impl(hape_join* h, const hape_relation* R, const hape_re
   res->n_items = (uint32_t)(r[5] & 0xFFFFFFFFu);
   fill_plan_fields(res, pl, loc[0].n, loc[1].n);
   res->exchange_path = h->xchg_path;
-  if (mat && out->mem == HAPE_MEM_HOST && res->n_written) {
-    CK(h, cudaMemcpyAsync(out->r_payload, mo.r, res->n_written * prw, cudaMemcpyDeviceToHost, h->stream));
-    CK(h, cudaMemcpyAsync(out->s_payload, mo.s, res->n_written * psw, cudaMemcpyDeviceToHost, h->stream));
+  if (host_pairs) {
+    if (res->n_written) {
+      CK(h, cudaMemcpyAsync(out->r_payload, mo.r, res->n_written * prw, cudaMemcpyDeviceToHost, h->stream));
+      CK(h, cudaMemcpyAsync(out->s_payload, mo.s, res->n_written * psw, cudaMemcpyDeviceToHost, h->stream));
+    }
+    cudaEventRecord(h->ev[HAPE_NSTAGES], h->stream);
+    CK(h, cudaStreamSynchronize(h->stream));
   }
-  cudaEventRecord(h->ev[HAPE_NSTAGES], h->stream);
-  CK(h, cudaStreamSynchronize(h->stream));
   res->kernel_launches = h->launches;
   stage_times(h, res);
   if (mat && r[4] > out->capacity)
