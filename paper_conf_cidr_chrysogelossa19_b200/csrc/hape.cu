@@ -81,7 +81,7 @@ struct hape_join {
   unsigned long long* h_res = nullptr;  // pinned: acc[4], out_ctr, (n_items | item_ctr)
   // cached CUDA graph of the local join sequence (keyed by pointers + sizes)
   cudaGraphExec_t gexec = nullptr;
-  uintptr_t gkey[16] = {};
+  uintptr_t gkey[18] = {};
   uint32_t g_launches = 0, g_join_ctas = 0;
   bool g_ev_used[HAPE_NSTAGES] = {};
   uint32_t* h_bounds = nullptr;         // pinned: gathered device-partition bounds
@@ -445,8 +445,9 @@ static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, 
   if (grid == 0) return HAPE_OK;
   // warp-aggregated ranking: always for narrow fan-outs (the destination
   // route, P <= 64: lanes share buckets), else HAPE_SC_AGG=1
+  // (wider fan-outs: HAPE_SC_AGG=1 match_any form, 2 the hot-bucket form)
   static const uint32_t agg_env = (uint32_t)env_int("HAPE_SC_AGG", 0);
-  const uint32_t agg = agg_env || P <= 64;
+  const uint32_t agg = P <= 64 ? 1u : agg_env;
   kern<<<grid, C::NT, smem, h->stream>>>(s.in, m, bf, P, offs, static_cast<Tup<KW, PW>*>(out), nullptr, agg,
                                          lk ? *lk : LinkMap{});
   CK_LAUNCH(h);
@@ -1385,7 +1386,7 @@ static hape_status local_join(hape_join* h, const Src loc_in[2], const MatOut& m
                              (uintptr_t)loc[1].in.t, (uintptr_t)loc[1].n,    (uintptr_t)mo.r,
                              (uintptr_t)mo.s,        (uintptr_t)(mo.on ? mo.cap : 0), (uintptr_t)h->small.p,
                              (uintptr_t)h->ping[0].p, (uintptr_t)h->ping[1].p, (uintptr_t)h->pong[0].p,
-                             (uintptr_t)h->pong[1].p};
+                             (uintptr_t)h->pong[1].p, (uintptr_t)h->lbuf[0].p, (uintptr_t)h->lbuf[1].p};
     static_assert(sizeof key == sizeof h->gkey, "graph key size");
     if (!h->gexec || memcmp(key, h->gkey, sizeof key) != 0) {
       if (h->gexec) { cudaGraphExecDestroy(h->gexec); h->gexec = nullptr; }

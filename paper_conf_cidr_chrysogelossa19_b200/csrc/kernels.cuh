@@ -863,6 +863,18 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
     // agg (skewed inputs): lanes of a warp that share a bucket rank through
     // one leader atomic (__match_any_sync) instead of
     // serialising on the same shared-memory word
+    // agg == 2 (hot-bucket form): the lanes whose bucket equals lane 0's
+    // rank through lane 0's one atomic (one shuffle + one ballot per tuple);
+    // a skewed tile's hot bucket holds lane 0 most of the time
+    auto rank_hot = [&](uint32_t b) -> uint32_t {
+      const uint32_t b0 = __shfl_sync(0xffffffffu, b, 0);
+      const uint32_t m = __ballot_sync(0xffffffffu, b == b0);
+      if (__popc(m) < 4) return atomicAdd(&s_cnt[b], 1u);
+      uint32_t base = 0;
+      if (lane == 0) base = atomicAdd(&s_cnt[b0], (uint32_t)__popc(m));
+      base = __shfl_sync(0xffffffffu, base, 0);
+      return b == b0 ? base + (uint32_t)__popc(m & ((1u << lane) - 1u)) : atomicAdd(&s_cnt[b], 1u);
+    };
     auto rank_agg = [&](uint32_t b, uint32_t mask) -> uint32_t {
       const uint32_t peers = __match_any_sync(mask, b);
       const int leader = __ffs(peers) - 1;
@@ -874,11 +886,17 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
     if (full) {
 #pragma unroll
       for (int u = 0; u < ITEMS; u++) x[u] = load(u * NT + threadIdx.x);
-      if (agg) {
+      if (agg == 1) {
 #pragma unroll
         for (int u = 0; u < ITEMS; u++) {
           const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
           br[u] = (b << 16) | rank_agg(b, 0xffffffffu);
+        }
+      } else if (agg == 2) {
+#pragma unroll
+        for (int u = 0; u < ITEMS; u++) {
+          const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
+          br[u] = (b << 16) | rank_hot(b);
         }
       } else {
 #pragma unroll
@@ -895,7 +913,7 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
         if (i < tn) {
           x[u] = load(i);
           const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
-          br[u] = (b << 16) | (agg ? rank_agg(b, vm) : atomicAdd(&s_cnt[b], 1u));
+          br[u] = (b << 16) | (agg == 1 ? rank_agg(b, vm) : atomicAdd(&s_cnt[b], 1u));
         }
       }
     }

@@ -519,3 +519,21 @@ def test_linked_partition_invariants(bits, kb):
     assert np.array_equal(ok, keys[op.astype(np.int64)])
     pid = partition.partition_id(ok, b1, b2)
     assert np.array_equal(pid, np.repeat(np.arange(Q), np.diff(ob)))
+
+
+def test_linked_graph_replay_after_workspace_regrowth():
+    """The cached CUDA graph of a linked join must not outlive the buffer
+    directory it captured: a larger debug partition on the same handle
+    regrows the directory, and the next join with the old pointers/sizes
+    must re-capture (graph key includes the directory)."""
+    j = RadixJoin(key_dtype=torch.int32, radix_passes=2, radix_bits=(8, 8), linked=True)
+    wl = datagen.make("c2", n_r=1 << 18, n_s=1 << 18)
+    args = [cuda(a) for a in (wl.R.key, wl.R.payload, wl.S.key, wl.S.payload)]
+    want = provenance.expected_from_workload(wl)
+    check(j.join(*args), want)
+    big = datagen.make("c2", n_r=1 << 21, n_s=1 << 21)
+    j.debug_partition(cuda(big.R.key), cuda(big.R.payload))
+    torch.cuda.empty_cache()
+    check(j.join(*args), want)
+    check(j.join(*args), want)
+    j.close()
