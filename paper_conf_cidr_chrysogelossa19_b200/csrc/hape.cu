@@ -509,26 +509,22 @@ static hape_status scatter_i(hape_join* h, const Src& s, SegMap m, BitField bf, 
                              void* out) {
   static int v = [] { const char* e = getenv("HAPE_SC"); return e ? atoi(e) : 0; }();
   // measured (round 1): 8-byte tuples <512,13,2,2> (C2 scatters 1.09/1.03 ->
-  // 0.96/0.93 ms vs the earlier <512,8,3,2>); 16-byte tuples <384,9,2,2>
-  // (C3 7.95/7.04 -> 7.10/6.89 ms vs <256,8,2,3>).  The largest tile two CTAs
-  // per SM can stage wins: longer bucket runs per tile (P585-589: more staged
-  // tuples per partition -> longer runs -> better store coalescing).
-  // HAPE_SC / HAPE_SC16 select the alternatives (tuning only).
+  // 0.96/0.93 ms vs <512,8,3,2>; <512,12,2,2> slower); 16-byte tuples
+  // <384,9,2,2> (C3 7.95/7.04 -> 7.10/6.89 ms vs <256,8,2,3>).  The largest
+  // tile two CTAs per SM can stage wins: longer bucket runs per tile
+  // (P585-589: more staged tuples per partition -> longer runs -> better
+  // store coalescing).  (The swept alternatives are no longer instantiated.)
   if constexpr (KW + PW <= 8) {
-    if (v == 1) return scatter_t<KW, PW, AOS, ScCfg<512, 8, 3, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
-    if (v == 2) return scatter_t<KW, PW, AOS, ScCfg<512, 12, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
     // wide fan-outs (>= 1024 buckets): one CTA per SM staging twice the tile
     // (longer runs per bucket and tile); HAPE_SC=3 forces it, used for P >= 1024 unless HAPE_SC_WIDE=0
-    // (measured C4 at N=1, 2 x 1024 buckets: scatters 25.0 / 23.3 -> 18.8 / 18.4 ms)
+    // (measured C4 at N=1, 2 x 1024 buckets: scatters 25.0 / 23.3 -> 18.8 / 18.4 ms;
+    // on 256 / 512 buckets it is slower: C2 0.94 -> 1.08 ms, C5 4.92 -> 5.43 ms)
     static int wide = [] { const char* e = getenv("HAPE_SC_WIDE"); return e ? atoi(e) : 1; }();
     using Cw = ScCfg<1024, 12, 2, 1>;
     if (v == 3 || (wide && P >= 1024 && ScLayout<KW, PW, AOS, Cw>::bytes(P) <= kScatterSmemMax))
       return scatter_t<KW, PW, AOS, Cw, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
     return scatter_t<KW, PW, AOS, ScCfg<512, 13, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
   } else {
-    static int w = [] { const char* e = getenv("HAPE_SC16"); return e ? atoi(e) : 0; }();
-    if (w == 1) return scatter_t<KW, PW, AOS, ScCfg<256, 8, 2, 3>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
-    if (w == 2) return scatter_t<KW, PW, AOS, ScCfg<256, 12, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
     return scatter_t<KW, PW, AOS, ScCfg<384, 9, 2, 2>, IDENT, CLAIM>(h, s, m, bf, P, offs, out);
   }
 }
@@ -649,33 +645,27 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
 template <int KW, int PRW, int PSW>
 static hape_status launch_join_m(hape_join* h, const JoinArgs& a, bool mat, uint32_t* ctas) {
   // S tile tuples per thread of the SR form (0 = direct S loads); consumer
-  // threads per CTA (HAPE_JN_NC=512: twice the warps per CTA)
+  // threads per CTA (SR: 512, direct: 256)
   // Measured (C3 build+probe): direct 14.1 ms; SR 256 threads, 1024-tuple
   // tiles 12.4; SR 512 threads, 1024-tuple tiles 10.7 ms.  C2 (8-byte tuples,
   // no pairs): direct 256 threads 0.74 ms, every SR / 512-thread form slower.
-  static const int su_env = env_int("HAPE_JN_SU", -1), nc_env = env_int("HAPE_JN_NC", 0);
-  const bool sr_form = mat || KW + PSW > 8;
-  const int su = su_env >= 0 ? su_env : (sr_form ? 2 : 0);
-  const bool wide = nc_env ? nc_env == 512 : sr_form;
-#define HAPE_JN_SU(M, NC)                                                  \
-  switch (su) {                                                            \
-    case 0: return launch_join_t<KW, PRW, PSW, M, 0, NC>(h, a, ctas);      \
-    case 1: return launch_join_t<KW, PRW, PSW, M, 1, NC>(h, a, ctas);      \
-    case 2: return launch_join_t<KW, PRW, PSW, M, 2, NC>(h, a, ctas);      \
-    default: return launch_join_t<KW, PRW, PSW, M, 4, NC>(h, a, ctas);     \
+  // (the swept SU = 1 / 4 depths and the 512-thread direct form are no
+  // longer instantiated; HAPE_JN_SU=2 forces the SR form, 0 the direct form)
+  static const int su_env = env_int("HAPE_JN_SU", -1);
+  const bool sr_form = su_env >= 0 ? su_env > 0 : (mat || KW + PSW > 8);
+  if (sr_form) {
+    if (mat) return launch_join_t<KW, PRW, PSW, true, 2, 512>(h, a, ctas);
+    return launch_join_t<KW, PRW, PSW, false, 2, 512>(h, a, ctas);
   }
-  if (wide) {
-    if (mat) { HAPE_JN_SU(true, 512) } else { HAPE_JN_SU(false, 512) }
-  }
-  if (mat) { HAPE_JN_SU(true, 256) } else { HAPE_JN_SU(false, 256) }
-#undef HAPE_JN_SU
+  if (mat) return launch_join_t<KW, PRW, PSW, true, 0, 256>(h, a, ctas);
+  return launch_join_t<KW, PRW, PSW, false, 0, 256>(h, a, ctas);
 }
 
 // Open-addressing build+probe (join_oa.cuh).  Shape: 256 threads for
 // 8-byte R tuples, 512 for 16-byte ones (the R chunk lives in registers:
 // OA_CAPMAX / NC tuples per thread); NTAB = 2 tables (one barrier per stage)
 // when two still fit 2+ CTAs per SM, else 1; U = 2 S tuples per thread per
-// batch.  HAPE_OA_NTAB / HAPE_OA_U / HAPE_OA_SB (extra slot bits) tune the
+// batch.  HAPE_OA_SB (extra slot bits) tunes the
 // int32 form.  HAPE_JN_OA=1 selects it (default: the chained k_build_probe).
 template <int KW, int PRW, int PSW, bool MAT, bool IDENT, int NC, int NTAB, int U>
 static hape_status launch_oa_t(hape_join* h, const JoinArgs& a_in, uint32_t* ctas_out) {
@@ -704,19 +694,9 @@ template <int KW, int PRW, int PSW, bool MAT, bool IDENT>
 static hape_status launch_oa_m(hape_join* h, const JoinArgs& a, uint32_t* ctas) {
   constexpr bool W8 = sizeof(Tup<KW, PRW>) == 8;
   constexpr int NC = W8 ? 256 : 512;
-  if constexpr (KW == 4 && PRW == 4 && PSW == 4 && !MAT && !IDENT) {
-    static const int ntab = env_int("HAPE_OA_NTAB", 2), u = env_int("HAPE_OA_U", 2);
-    if (ntab == 1) {
-      if (u == 1) return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, 1, 1>(h, a, ctas);
-      if (u == 4) return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, 1, 4>(h, a, ctas);
-      return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, 1, 2>(h, a, ctas);
-    }
-    if (u == 1) return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, 2, 1>(h, a, ctas);
-    if (u == 4) return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, 2, 4>(h, a, ctas);
-    return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, 2, 2>(h, a, ctas);
-  } else {
-    return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, W8 ? 2 : 1, 2>(h, a, ctas);
-  }
+  // (measured shapes, C2: NTAB 1 3.81 / 2 4.03 ms, U 1 / 2 / 4 within 1 %;
+  // only the default is instantiated)
+  return launch_oa_t<KW, PRW, PSW, MAT, IDENT, NC, W8 ? 2 : 1, 2>(h, a, ctas);
 }
 
 template <int KW, int PRW, int PSW>
