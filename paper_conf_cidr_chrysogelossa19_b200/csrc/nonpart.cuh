@@ -55,6 +55,45 @@ __device__ __forceinline__ uint32_t np_slot(typename UW<KW>::T k, uint32_t mask)
 
 constexpr int NP_THREADS = 256;
 
+// one claim attempt of an insert at slot s: true when the tuple now owns it
+template <int KW, int PW>
+__device__ __forceinline__ bool np_try(NpSlot<KW, PW>* __restrict__ tab, uint32_t s, typename UW<KW>::T k,
+                                       typename UW<PW>::T p) {
+  if constexpr (sizeof(NpSlot<KW, PW>) == 16) {
+    // 16-byte slots: the whole slot (tag set) in one 128-bit compare-and-swap
+    // against an empty slot -- one memory operation per insert attempt
+    NpSlot<KW, PW> v{};
+    v.key = k;
+    v.pay = p;
+    v.tag = 1;
+    const ulonglong2 nv = *reinterpret_cast<const ulonglong2*>(&v);
+    unsigned long long olo, ohi;
+    asm volatile(
+        "{\n .reg .b128 d, b, c;\n mov.b128 b, {%2, %3};\n mov.b128 c, {%4, %5};\n"
+        " atom.global.cas.b128 d, [%6], b, c;\n mov.b128 {%0, %1}, d;\n}"
+        : "=l"(olo), "=l"(ohi)
+        : "l"(0ull), "l"(0ull), "l"(nv.x), "l"(nv.y), "l"(tab + s)
+        : "memory");
+    return olo == 0ull && ohi == 0ull;
+  } else {
+    if (atomicCAS(&tab[s].tag, 0u, 1u) != 0u) return false;
+    if constexpr (KW == 8 && PW == 8) {
+      *reinterpret_cast<ulonglong2*>(&tab[s]) = make_ulonglong2(k, p);
+    } else {
+      tab[s].key = k;
+      tab[s].pay = p;
+    }
+    return true;
+  }
+}
+
+// NP_U probes per thread in flight (C2 probe 4.74 -> 4.37 ms).  The build
+// stays one insert at a time: four independent 128-bit CAS per thread
+// measured 13.2 vs 12.1 ms -- the inserts are bound by random atomics into
+// the 4 GB table (a read-modify-write of a random DRAM sector each), not by
+// latency.
+constexpr int NP_U = 4;
+
 template <int KW, int PW>
 __global__ void __launch_bounds__(NP_THREADS)
 k_np_build(const typename UW<KW>::T* __restrict__ rk, const typename UW<PW>::T* __restrict__ rp, uint32_t n,
@@ -63,34 +102,7 @@ k_np_build(const typename UW<KW>::T* __restrict__ rk, const typename UW<PW>::T* 
     const typename UW<KW>::T k = rk[i];
     const typename UW<PW>::T p = rp[i];
     uint32_t s = np_slot<KW>(k, mask);
-    if constexpr (sizeof(NpSlot<KW, PW>) == 16) {
-      // 16-byte slots: the whole slot (tag set) in one 128-bit compare-and-swap
-      // against an empty slot -- one memory operation per insert attempt
-      NpSlot<KW, PW> v{};
-      v.key = k;
-      v.pay = p;
-      v.tag = 1;
-      const ulonglong2 nv = *reinterpret_cast<const ulonglong2*>(&v);
-      while (true) {
-        unsigned long long olo, ohi;
-        asm volatile(
-            "{\n .reg .b128 d, b, c;\n mov.b128 b, {%2, %3};\n mov.b128 c, {%4, %5};\n"
-            " atom.global.cas.b128 d, [%6], b, c;\n mov.b128 {%0, %1}, d;\n}"
-            : "=l"(olo), "=l"(ohi)
-            : "l"(0ull), "l"(0ull), "l"(nv.x), "l"(nv.y), "l"(tab + s)
-            : "memory");
-        if (olo == 0ull && ohi == 0ull) break;
-        s = (s + 1) & mask;
-      }
-      continue;
-    }
-    while (atomicCAS(&tab[s].tag, 0u, 1u) != 0u) s = (s + 1) & mask;
-    if constexpr (KW == 8 && PW == 8) {
-      *reinterpret_cast<ulonglong2*>(&tab[s]) = make_ulonglong2(k, p);
-    } else {
-      tab[s].key = k;
-      tab[s].pay = p;
-    }
+    while (!np_try<KW, PW>(tab, s, k, p)) s = (s + 1) & mask;
   }
 }
 
@@ -164,37 +176,45 @@ k_np_probe(const typename UW<KW>::T* __restrict__ sk, const typename UW<PSW>::T*
       __syncthreads();  // s_c / s_base are reused by the next batch
     }
   } else {
-    const uint32_t nwarps = gridDim.x * (NP_THREADS / 32);
-    // warp-uniform loop: every lane of a warp runs the same iterations; a
-    // lane walks to its next match, the aggregation runs converged per round
-    for (uint32_t base = (blockIdx.x * (NP_THREADS / 32) + warp) * 32u; base < n; base += nwarps * 32u) {
-      const uint32_t j = base + lane;
-      bool active = j < n;
-      typename UW<KW>::T k{};
-      int64_t q = 0;
-      uint32_t s = 0;
-      if (active) {
-        k = sk[j];
-        q = (int64_t)(PS)sp[j];
-        s = np_slot<KW>(k, mask);
-      }
-      while (__any_sync(0xffffffffu, active)) {
-        bool hit = false;
-        int64_t p = 0;
-        if (active) {
-          while (true) {
-            const NpSlot<KW, PRW> e = np_load(tab + s);
-            if (!e.tag) { active = false; break; }
-            s = (s + 1) & mask;
-            if (e.key == k) { hit = true; p = (int64_t)(PR)e.pay; break; }
-          }
+    // NP_U S tuples per thread: their first slot loads are issued together
+    // (independent random HBM reads in flight), then each walks on from its
+    // loaded slot to the first empty one (or its first match, unique R)
+    for (uint32_t base = blockIdx.x * NP_THREADS * NP_U + threadIdx.x; base < n;
+         base += gridDim.x * NP_THREADS * NP_U) {
+      typename UW<KW>::T k[NP_U];
+      int64_t q[NP_U];
+      uint32_t sl[NP_U];
+      NpSlot<KW, PRW> e[NP_U];
+      bool v[NP_U];
+#pragma unroll
+      for (int u = 0; u < NP_U; u++) {
+        const uint32_t j = base + u * NP_THREADS;
+        v[u] = j < n;
+        if (v[u]) {
+          k[u] = sk[j];
+          q[u] = (int64_t)(PS)sp[j];
+          sl[u] = np_slot<KW>(k[u], mask);
         }
-        if (hit) {
-          cnt++;
-          sr += (unsigned long long)p;
-          ss += (unsigned long long)q;
-          sx += pair_mix(p, q);
-          if (r_unique) active = false;
+      }
+#pragma unroll
+      for (int u = 0; u < NP_U; u++)
+        if (v[u]) e[u] = np_load(tab + sl[u]);
+#pragma unroll
+      for (int u = 0; u < NP_U; u++) {
+        if (!v[u]) continue;
+        uint32_t s = sl[u];
+        NpSlot<KW, PRW> x = e[u];
+        while (x.tag) {
+          if (x.key == k[u]) {
+            const int64_t p = (int64_t)(PR)x.pay;
+            cnt++;
+            sr += (unsigned long long)p;
+            ss += (unsigned long long)q[u];
+            sx += pair_mix(p, q[u]);
+            if (r_unique) break;
+          }
+          s = (s + 1) & mask;
+          x = np_load(tab + s);
         }
       }
     }
