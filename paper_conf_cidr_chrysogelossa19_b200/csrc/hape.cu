@@ -216,6 +216,14 @@ static hape_status make_plan(const hape_join* h, uint64_t n_r, uint64_t n_s, hap
   p->dest_bits = ceil_log2_u64((uint64_t)world);
   uint32_t need = 0;
   while ((n_r >> need) > kTargetPerPartition) need++;
+  // a 17-bit plan would lose the one-read joint histogram of both passes
+  // (k_hist_joint counts at most 2^16 joint buckets); one bit less keeps it,
+  // at ~4096 R tuples per co-partition -- worth it while S is not much larger
+  // than R (measured: C4's 2^28-per-rank share 6.46 -> 6.24 ms; C5, |S| = 4|R|,
+  // 16.61 -> 17.42 ms at theta 0.5: the larger co-partitions cost the probe
+  // more than the histogram read saves).  HAPE_PLAN16=0: plain 17-bit plans.
+  static const int plan16 = env_int("HAPE_PLAN16", 1);
+  if (plan16 && need == 17 && n_s <= 2 * n_r && !c.radix_passes && !c.radix_bits[0]) need = 16;
   uint32_t passes = c.radix_passes ? (uint32_t)c.radix_passes : (need <= kMaxSinglePassBits ? 1u : 2u);
   uint32_t b1, b2;
   if (c.radix_bits[0] > 0) {
