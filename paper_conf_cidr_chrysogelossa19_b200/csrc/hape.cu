@@ -1878,7 +1878,7 @@ hape_status hape_join_create(const hape_join_config* cfg, hape_join** out_handle
       cfg->radix_bits[1] > (int)kMaxBitsPerPass)
     return HAPE_ERR_INVALID_ARG;
   const int world = cfg->world_size > 1 ? cfg->world_size : 1;
-  if (cfg->world_size < 0 || (world & (world - 1)) != 0) return HAPE_ERR_INVALID_ARG;
+  if (cfg->world_size < 0 || (world & (world - 1)) != 0 || world > 64) return HAPE_ERR_INVALID_ARG;
   if (cfg->rank < 0 || cfg->rank >= world) return HAPE_ERR_INVALID_ARG;
   if (world > 1 && !cfg->nccl_comm) return HAPE_ERR_INVALID_ARG;
   if (cfg->device < 0) return HAPE_ERR_INVALID_ARG;

@@ -54,7 +54,7 @@ def test_status_strings(lib):
 
 def test_create_rejects_bad_config_without_touching_cuda(lib):
     for field, val in (("key_type", 7), ("radix_passes", 3), ("part_fn", 5), ("world_size", 3),
-                       ("device", -1)):
+                       ("world_size", 128), ("device", -1), ("flags", 4)):
         cfg = lib.hape_join_config()
         setattr(cfg, field, val)
         st, h = lib.hape_join_create(cfg)
