@@ -1349,6 +1349,9 @@ static hape_status local_join(hape_join* h, const Src loc_in[2], const MatOut& m
     ja.items = at<uint2>(h, L.items); ja.n_items = ctrs;
     ja.cap = pl.build_cap; ja.slice = pl.probe_slice; ja.slot_bits = pl.slot_bits;
     ja.qmask = Q - 1;
+    // (HAPE_JN_EPOCH_PERIOD: test-only, forces frequent head resets)
+    static const int ep_env = env_int("HAPE_JN_EPOCH_PERIOD", 65535);
+    ja.ep_period = (uint32_t)std::max(1, std::min(65535, ep_env));
     ja.acc = at<unsigned long long>(h, L.acc);
     ja.out_r = mo.r; ja.out_s = mo.s; ja.out_cap = mo.on ? mo.cap : 0;
     ja.out_ctr = at<unsigned long long>(h, L.out_ctr);

@@ -1172,6 +1172,7 @@ struct JoinArgs {
   uint32_t nrb;                              // R-chunk ring buffers (1 or 2)
   uint32_t nsb;                              // SR kernels: staged S tiles in the ring (>= 2)
   uint32_t qmask;                            // co-partitions - 1: q = h(key) & qmask (k_join_oa)
+  uint32_t ep_period;                        // chain-head epochs before a head reset (<= 65535)
 };
 
 struct JnStage {
@@ -1453,11 +1454,11 @@ k_build_probe(JoinArgs a) {
     uint32_t sseq = 0;
     for (uint32_t stage = 0;; stage++) {
       const uint32_t bi = stage % NRB, ph = (stage / NRB) & 1;
-      // stage epoch (1..65535): heads of other epochs read as empty chains,
-      // so the table needs no reset; every 65535 stages the heads are zeroed
-      // (epoch 0 is never used) -- the previous stage's probe is complete
-      // (barrier at the end of the loop body)
-      const uint32_t ep = stage % 65535u + 1u;
+      // stage epoch (1..ep_period, ep_period <= 65535): heads of other
+      // epochs read as empty chains, so the table needs no reset; every
+      // ep_period stages the heads are zeroed (epoch 0 is never used) -- the
+      // previous stage's probe is complete (barrier at the end of the loop body)
+      const uint32_t ep = stage % a.ep_period + 1u;
       if (ep == 1u && stage > 0) {
         for (uint32_t i = threadIdx.x * 4; i < nslots; i += JN_CONSUMERS * 4)
           *reinterpret_cast<uint4*>(s_head + i) = make_uint4(0u, 0u, 0u, 0u);
