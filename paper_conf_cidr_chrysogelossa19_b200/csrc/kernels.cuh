@@ -1360,8 +1360,12 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
 // consumers never wait on HBM latency -- the form for materialising and
 // 16-byte-tuple joins, whose probe cannot keep a software-pipelined S batch
 // in registers.
+// (HAPE_JN_MINB: CTAs per SM the direct form is register-budgeted for; A/B builds)
+#ifndef HAPE_JN_MINB
+#define HAPE_JN_MINB 1
+#endif
 template <int KW, int PRW, int PSW, bool MAT, int SU, int JN_CONSUMERS = 256>
-__global__ void __launch_bounds__(JN_CONSUMERS + 32)
+__global__ void __launch_bounds__(JN_CONSUMERS + 32, SU == 0 ? HAPE_JN_MINB : 1)
 k_build_probe(JoinArgs a) {
   constexpr int JN_THREADS = JN_CONSUMERS + 32;
   constexpr bool SR = SU > 0;
