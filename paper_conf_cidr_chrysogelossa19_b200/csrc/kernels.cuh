@@ -1360,12 +1360,21 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
 // consumers never wait on HBM latency -- the form for materialising and
 // 16-byte-tuple joins, whose probe cannot keep a software-pipelined S batch
 // in registers.
-// (HAPE_JN_MINB: CTAs per SM the direct form is register-budgeted for; A/B builds)
+// (HAPE_JN_MINB / HAPE_JN_SR_MINB: CTAs per SM the direct / staged-S forms
+// are register-budgeted for; A/B builds)
 #ifndef HAPE_JN_MINB
-#define HAPE_JN_MINB 1
+// the direct form (8-byte S tuples, no pairs) at 4 CTAs per SM: <= 56
+// registers, no spills; unbounded it took 63 (3 CTAs per SM: C2 0.78 vs 0.74 ms)
+#define HAPE_JN_MINB 4
+#endif
+#ifndef HAPE_JN_SR_MINB
+// the staged-S form needs 2 CTAs per SM: unbounded it took 72 registers (one
+// 544-thread CTA per SM, 36 % barrier stalls): C3 build+probe 15.3 vs 10.6 ms
+#define HAPE_JN_SR_MINB 2
 #endif
 template <int KW, int PRW, int PSW, bool MAT, int SU, int JN_CONSUMERS = 256>
-__global__ void __launch_bounds__(JN_CONSUMERS + 32, SU == 0 ? HAPE_JN_MINB : 1)
+__global__ void __launch_bounds__(JN_CONSUMERS + 32,
+                                  SU == 0 ? ((KW + PSW <= 8 && !MAT) ? HAPE_JN_MINB : 1) : HAPE_JN_SR_MINB)
 k_build_probe(JoinArgs a) {
   constexpr int JN_THREADS = JN_CONSUMERS + 32;
   constexpr bool SR = SU > 0;
@@ -1455,14 +1464,14 @@ k_build_probe(JoinArgs a) {
     }
   } else {
     // ------------------------------ consumer warps -----------------------------
-    uint32_t sseq = 0;
+    uint32_t sseq = 0, ep = 0;
     for (uint32_t stage = 0;; stage++) {
       const uint32_t bi = stage % NRB, ph = (stage / NRB) & 1;
       // stage epoch (1..ep_period, ep_period <= 65535): heads of other
       // epochs read as empty chains, so the table needs no reset; every
       // ep_period stages the heads are zeroed (epoch 0 is never used) -- the
       // previous stage's probe is complete (barrier at the end of the loop body)
-      const uint32_t ep = stage % a.ep_period + 1u;
+      if (++ep > a.ep_period) ep = 1u;
       if (ep == 1u && stage > 0) {
         for (uint32_t i = threadIdx.x * 4; i < nslots; i += JN_CONSUMERS * 4)
           *reinterpret_cast<uint4*>(s_head + i) = make_uint4(0u, 0u, 0u, 0u);
