@@ -1150,12 +1150,15 @@ __host__ __device__ constexpr size_t join_stile_bytes() {
 }
 // nrb R-chunk buffers, nsb staged S tiles of SU*256 tuples (SU = 0: S read
 // straight from HBM)
-template <int KW, int PRW, int PSW, int SU = 0, int NC = 256>
+// KN (key|next nodes): the build moves each R payload to pay[] and stores
+// the chain link in the tuple's payload field, so a chain hop is one shared
+// load of {key, next}; otherwise a u16 next[] array beside the tuples
+template <int KW, int PRW, int PSW, int SU = 0, int NC = 256, bool KN = false>
 __host__ __device__ constexpr size_t join_smem_bytes(uint32_t cap, uint32_t slot_bits, uint32_t nrb = 2,
                                                      uint32_t nsb = 0) {
   return nrb * join_ring_bytes<KW, PRW>(cap)                               // R ring
          + (SU ? nsb * join_stile_bytes<KW, PSW, SU, NC>() : 0)           // S ring
-         + ((size_t)cap * 2 + 15) / 16 * 16                                // next[]
+         + ((size_t)cap * (KN ? PRW : 2) + 15) / 16 * 16                   // pay[] / next[]
          + (sizeof(JnHead) << slot_bits);                                  // heads[]
 }
 
@@ -1197,14 +1200,33 @@ struct JnAcc {
   unsigned long long cnt = 0, sr = 0, ss = 0, sx = 0;
 };
 
-template <int KW, int PRW>
+template <int KW, int PRW, bool KN = false>
 struct JnTable {
-  const Tup<KW, PRW>* r;    // R chunk (ring buffer)
-  const uint16_t* next;
+  using V = typename UW<PRW>::T;
+  const Tup<KW, PRW>* r;    // R chunk (ring buffer); KN: {key, next} nodes
+  const void* link;         // next[] (u16), or KN: pay[] (the R payloads)
   const JnHead* head;
   uint32_t sbits;
   bool dup;                 // the chunk holds some key twice (bag semantics path)
   uint32_t ep;              // stage epoch: a head is valid iff its high half == ep
+  // chain successor of e, whose tuple y = r[e] is already loaded
+  __device__ __forceinline__ uint32_t next_of(uint32_t e, const Tup<KW, PRW>& y) const {
+    if constexpr (KN) return (uint32_t)y.v;
+    else return static_cast<const uint16_t*>(link)[e];
+  }
+  __device__ __forceinline__ uint32_t next_at(uint32_t e) const {
+    if constexpr (KN) return (uint32_t)r[e].v;
+    else return static_cast<const uint16_t*>(link)[e];
+  }
+  // R payload of e (y = r[e] already loaded)
+  __device__ __forceinline__ V pay_of(uint32_t e, const Tup<KW, PRW>& y) const {
+    if constexpr (KN) return static_cast<const V*>(link)[e];
+    else return y.v;
+  }
+  __device__ __forceinline__ V pay_at(uint32_t e) const {
+    if constexpr (KN) return static_cast<const V*>(link)[e];
+    else return r[e].v;
+  }
 };
 
 // chain head of a slot: (epoch << 16) | tuple index; a head written in an
@@ -1226,8 +1248,8 @@ __device__ __forceinline__ void jn_load_batch(const JoinArgs& a, uint32_t base, 
 }
 
 // Probe the U S tuples x[] (loaded by jn_load_batch for the same base).
-template <int KW, int PRW, int PSW, bool MAT, int U, int JN_CONSUMERS>
-__device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const JoinArgs& a, uint32_t base,
+template <int KW, int PRW, int PSW, bool MAT, int U, int JN_CONSUMERS, bool KN>
+__device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, KN>& t, const JoinArgs& a, uint32_t base,
                                                uint32_t s_hi, const Tup<KW, PSW> (&x)[U], JnAcc& acc,
                                                uint32_t* s_wsum, unsigned long long* s_wbase) {
   using PR = typename UW<PRW>::S;
@@ -1256,10 +1278,10 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
       while (e != JN_NIL) {
         y = t.r[e];
         if (y.k == x[u].k) break;
-        e = t.next[e];
+        e = t.next_of(e, y);
       }
       if (e != JN_NIL) {
-        const int64_t pr = (int64_t)(PR)y.v, ps = (int64_t)(PS)x[u].v;
+        const int64_t pr = (int64_t)(PR)t.pay_of(e, y), ps = (int64_t)(PS)x[u].v;
         if (MAT) m[u] = e;
         c[u] = 1;
         acc.sr += (unsigned long long)pr;
@@ -1272,18 +1294,18 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
         while (e != JN_NIL) {
           y = t.r[e];
           if (y.k == x[u].k) break;
-          e = t.next[e];
+          e = t.next_of(e, y);
         }
         const bool hit = e != JN_NIL;
         if (!__any_sync(0xffffffffu, hit)) break;
         if (hit) {
-          const int64_t pr = (int64_t)(PR)y.v, ps = (int64_t)(PS)x[u].v;
+          const int64_t pr = (int64_t)(PR)t.pay_of(e, y), ps = (int64_t)(PS)x[u].v;
           if (MAT && c[u] == 0) m[u] = e;
           c[u]++;
           acc.sr += (unsigned long long)pr;
           acc.ss += (unsigned long long)ps;
           acc.sx += pair_mix(pr, ps);
-          e = t.next[e];
+          e = t.next_of(e, y);
         }
       }
     }
@@ -1331,7 +1353,7 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
         if (!c[u]) continue;
         const unsigned long long pos = wb + before[u] + incl[u] - 1;
         if (pos < a.out_cap) {
-          static_cast<PR*>(a.out_r)[pos] = (PR)t.r[m[u]].v;
+          static_cast<PR*>(a.out_r)[pos] = (PR)t.pay_at(m[u]);
           static_cast<PS*>(a.out_s)[pos] = (PS)x[u].v;
         }
       }
@@ -1341,10 +1363,10 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
     for (int u = 0; u < U; u++) {
       if (!c[u]) continue;
       unsigned long long pos = wb + before[u] + incl[u] - c[u];
-      for (uint32_t e = e0[u]; e != JN_NIL; e = t.next[e]) {
+      for (uint32_t e = e0[u]; e != JN_NIL; e = t.next_at(e)) {
         if (t.r[e].k == x[u].k) {
           if (pos < a.out_cap) {
-            static_cast<PR*>(a.out_r)[pos] = (PR)t.r[e].v;
+            static_cast<PR*>(a.out_r)[pos] = (PR)t.pay_at(e);
             static_cast<PS*>(a.out_s)[pos] = (PS)x[u].v;
           }
           pos++;
@@ -1372,7 +1394,7 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW>& t, const 
 // 544-thread CTA per SM, 36 % barrier stalls): C3 build+probe 15.3 vs 10.6 ms
 #define HAPE_JN_SR_MINB 2
 #endif
-template <int KW, int PRW, int PSW, bool MAT, int SU, int JN_CONSUMERS = 256>
+template <int KW, int PRW, int PSW, bool MAT, int SU, int JN_CONSUMERS = 256, bool KN = false>
 __global__ void __launch_bounds__(JN_CONSUMERS + 32,
                                   SU == 0 ? ((KW + PSW <= 8 && !MAT) ? HAPE_JN_MINB : 1) : HAPE_JN_SR_MINB)
 k_build_probe(JoinArgs a) {
@@ -1387,9 +1409,9 @@ k_build_probe(JoinArgs a) {
   const uint32_t NRB = a.nrb, NSB = SR ? a.nsb : 0u;
   unsigned char* ring = smem;                                           // [NRB][RB]
   unsigned char* sring = smem + NRB * RB;                               // [NSB][SB]
-  uint16_t* s_next = reinterpret_cast<uint16_t*>(sring + NSB * SB);
-  JnHead* s_head = reinterpret_cast<JnHead*>(reinterpret_cast<unsigned char*>(s_next) +
-                                                 ((size_t)a.cap * 2 + 15) / 16 * 16);
+  uint16_t* s_next = reinterpret_cast<uint16_t*>(sring + NSB * SB);               // !KN
+  typename UW<PRW>::T* s_pay = reinterpret_cast<typename UW<PRW>::T*>(sring + NSB * SB);  // KN
+  JnHead* s_head = reinterpret_cast<JnHead*>(sring + NSB * SB + ((size_t)a.cap * (KN ? PRW : 2) + 15) / 16 * 16);
   constexpr int MAXS = 8;
   __shared__ JnStage s_meta[2];
   __shared__ uint32_t s_soff[MAXS];
@@ -1491,14 +1513,29 @@ k_build_probe(JoinArgs a) {
       constexpr bool PIPE = !MAT && !SR;
       Tup<KW, PSW> xs[JN_U];
       if (PIPE && st.s_lo + BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, st.s_lo, st.s_hi, xs);
-      if (!(a.dbg & 4u))
-        for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
-          s_next[i] = (uint16_t)jn_head(atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], (ep << 16) | i), ep);
+      if (!(a.dbg & 4u)) {
+        if constexpr (KN) {
+          // the payload moves to pay[i], the link takes its place in the node
+          TR* rw = reinterpret_cast<TR*>(ring + bi * RB + st.off);
+          for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS) {
+            const TR y = rw[i];
+            const uint32_t nx = jn_head(atomicExch(&s_head[jn_slot<KW>(y.k, a.slot_bits)], (ep << 16) | i), ep);
+            s_pay[i] = y.v;
+            rw[i].v = (typename UW<PRW>::T)nx;
+          }
+          // generic-proxy writes into a buffer the bulk-copy engine refills
+          asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+        } else {
+          for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
+            s_next[i] = (uint16_t)jn_head(atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], (ep << 16) | i), ep);
+        }
+      }
       consumer_sync<JN_CONSUMERS>();
       // ---- probe (a12): stream the S slice.  Bag semantics walk every chain
       // to its end; a caller-declared unique build side (HAPE_FLAG_R_UNIQUE, a
       // primary key) stops at the first match.
-      const JnTable<KW, PRW> tab{r, s_next, s_head, a.slot_bits, a.r_unique == 0, ep};
+      const JnTable<KW, PRW, KN> tab{r, KN ? static_cast<const void*>(s_pay) : static_cast<const void*>(s_next),
+                                     s_head, a.slot_bits, a.r_unique == 0, ep};
       if constexpr (SR) {
         // staged S tiles: wait for the tile, copy this thread's tuples to
         // registers, release the tile (one arrival per warp), probe
@@ -1522,7 +1559,7 @@ k_build_probe(JoinArgs a) {
             consumer_sync<JN_CONSUMERS>();
             if (threadIdx.x == 0) mbar_arrive(&sempty[sb]);
           }
-          jn_probe_batch<KW, PRW, PSW, MAT, XU, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+          jn_probe_batch<KW, PRW, PSW, MAT, XU, JN_CONSUMERS, KN>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
         }
       } else {
         // Full batches are software pipelined (PIPE): batch b+1 is loaded into
@@ -1537,7 +1574,7 @@ k_build_probe(JoinArgs a) {
           } else {
             jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, base, st.s_hi, x);
           }
-          jn_probe_batch<KW, PRW, PSW, MAT, JN_U, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+          jn_probe_batch<KW, PRW, PSW, MAT, JN_U, JN_CONSUMERS, KN>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
           base += BATCH;
         }
         // ragged tail (< BATCH tuples, any JN_U): 4-, 2- and 1-wide batches
@@ -1547,17 +1584,17 @@ k_build_probe(JoinArgs a) {
           if (rem > 2 * JN_CONSUMERS) {
             Tup<KW, PSW> x[4];
             jn_load_batch<KW, PSW, 4, JN_CONSUMERS>(a, base, st.s_hi, x);
-            jn_probe_batch<KW, PRW, PSW, MAT, 4, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+            jn_probe_batch<KW, PRW, PSW, MAT, 4, JN_CONSUMERS, KN>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
             base += 4 * JN_CONSUMERS;
           } else if (rem > JN_CONSUMERS) {
             Tup<KW, PSW> x[2];
             jn_load_batch<KW, PSW, 2, JN_CONSUMERS>(a, base, st.s_hi, x);
-            jn_probe_batch<KW, PRW, PSW, MAT, 2, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+            jn_probe_batch<KW, PRW, PSW, MAT, 2, JN_CONSUMERS, KN>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
             base += 2 * JN_CONSUMERS;
           } else {
             Tup<KW, PSW> x[1];
             jn_load_batch<KW, PSW, 1, JN_CONSUMERS>(a, base, st.s_hi, x);
-            jn_probe_batch<KW, PRW, PSW, MAT, 1, JN_CONSUMERS>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+            jn_probe_batch<KW, PRW, PSW, MAT, 1, JN_CONSUMERS, KN>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
             base += JN_CONSUMERS;
           }
         }

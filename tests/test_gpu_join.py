@@ -421,14 +421,18 @@ def test_open_addressing_refill_cases(identity):
                                  dict(HAPE_HJ_TMA="1"), dict(HAPE_SC="3"), dict(HAPE_SC_WIDE="0"),
                                  dict(HAPE_JN_OA="1"), dict(HAPE_JN_SU="2"), dict(HAPE_JN_SU="0"),
                                  dict(HAPE_SC_AGG="1"), dict(HAPE_SC_AGG="2"),
-                                 dict(HAPE_JN_EPOCH_PERIOD="1"), dict(HAPE_JN_EPOCH_PERIOD="3")])
+                                 dict(HAPE_JN_EPOCH_PERIOD="1"), dict(HAPE_JN_EPOCH_PERIOD="3"),
+                                 dict(HAPE_JN_KN="1"), dict(HAPE_JN_KN="0"), dict(HAPE_JN_KN="1", HAPE_JN_SU="0"),
+                                 dict(HAPE_JN_KN="1", HAPE_JN_EPOCH_PERIOD="1")])
 def test_alternative_kernel_forms_vs_oracle(env):
     # the retained alternatives, each read once per process (child process):
     # HAPE_JOINT=0 the per-pass totals + claiming scatters (the path of plans
     # with bits[0]+bits[1] > 16), HAPE_CLAIM=0 per-CTA offset scatters,
     # HAPE_JN_OA=1 the open-addressing build+probe, HAPE_JN_SU the staged-S /
     # direct build+probe forms, HAPE_SC_AGG the warp-aggregated rankings,
-    # HAPE_JN_EPOCH_PERIOD the chain-head epoch wrap (reset every 1 / 3 stages)
+    # HAPE_JN_EPOCH_PERIOD the chain-head epoch wrap (reset every 1 / 3 stages),
+    # HAPE_JN_KN the key|next node table of the direct build+probe (default
+    # for bag semantics only) forced on / off
     import subprocess
     import sys
     import os
