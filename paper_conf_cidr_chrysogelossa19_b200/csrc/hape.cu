@@ -602,11 +602,11 @@ static hape_status launch_peer_scatter(hape_join* h, int kw, const Src& s, SegMa
 // straight from HBM with a register-pipelined batch.  HAPE_JN_SU=0/1/2/4
 // forces the form, HAPE_JN_NRB / HAPE_JN_NSB the ring depths (tuning only).
 
-template <int KW, int PRW, int PSW, bool MAT, int SU, int NC = 256, bool KN = false>
+template <int KW, int PRW, int PSW, bool MAT, int SU, int NC = 256, int LAY = JN_AOS>
 static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* ctas_out) {
   constexpr bool SR = SU > 0;
   constexpr int JN_THREADS = NC + 32;
-  auto kern = k_build_probe<KW, PRW, PSW, MAT, SU, NC, KN>;
+  auto kern = k_build_probe<KW, PRW, PSW, MAT, SU, NC, LAY>;
   JoinArgs a = a_in;
   static const int nrb_env = env_int("HAPE_JN_NRB", 0), nsb_env = env_int("HAPE_JN_NSB", 0);
   a.nsb = SR ? (uint32_t)std::min(8, std::max(2, nsb_env ? nsb_env : (SU >= 4 ? 3 : 2))) : 0u;
@@ -614,7 +614,7 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
   static uint64_t attr_dev = 0;
   CKS(smem_attr(h, kern, 200 * 1024, attr_dev));
   auto occ = [&](uint32_t sb, uint32_t nrb, int* per_sm) -> hape_status {
-    const size_t smem = join_smem_bytes<KW, PRW, PSW, SU, NC, KN>(a.cap, sb, nrb, a.nsb);
+    const size_t smem = join_smem_bytes<KW, PRW, PSW, SU, NC, LAY>(a.cap, sb, nrb, a.nsb);
     *per_sm = 0;
     if (smem > 200 * 1024) return HAPE_OK;
     CK(h, cudaOccupancyMaxActiveBlocksPerMultiprocessor(per_sm, kern, JN_THREADS, smem));
@@ -626,7 +626,7 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
   // other resident CTAs cover the R load at a stage boundary).  The direct
   // form also takes a single R buffer when that buys a larger head array at
   // the same occupancy (C2: 2^12 heads instead of 2^11, 4 CTAs per SM either
-  // way -- build+probe 0.742 -> 0.717 ms, profiles/r2/ab_kn.jsonl); shorter
+  // way -- build+probe 0.742 -> 0.717 ms, profiles/r2/ab_build_probe_nrb.jsonl); shorter
   // chains are worth more than covering the R load of a stage boundary
   if (!nrb_env && a.nrb == 2) {
     int p1 = 0;
@@ -641,7 +641,7 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
   }
   if (per_sm < 1)
     return fail(h, HAPE_ERR_UNSUPPORTED, "build+probe does not fit: smem %zu",
-                join_smem_bytes<KW, PRW, PSW, SU, NC, KN>(a.cap, a.slot_bits, a.nrb, a.nsb));
+                join_smem_bytes<KW, PRW, PSW, SU, NC, LAY>(a.cap, a.slot_bits, a.nrb, a.nsb));
   // plan.slot_bits is the minimum table size: one more bit (shorter chains)
   // when the larger head array costs no occupancy (register-limited kernels)
   while (a.slot_bits < 14) {
@@ -650,7 +650,7 @@ static hape_status launch_join_t(hape_join* h, const JoinArgs& a_in, uint32_t* c
     if (per_sm2 != per_sm) break;
     a.slot_bits = a.slot_bits + 1;
   }
-  const size_t smem_used = join_smem_bytes<KW, PRW, PSW, SU, NC, KN>(a.cap, a.slot_bits, a.nrb, a.nsb);
+  const size_t smem_used = join_smem_bytes<KW, PRW, PSW, SU, NC, LAY>(a.cap, a.slot_bits, a.nrb, a.nsb);
   const unsigned grid = (unsigned)(per_sm * h->num_sms);
   *ctas_out = grid;
   kern<<<grid, JN_THREADS, smem_used, h->stream>>>(a);
@@ -673,16 +673,21 @@ static hape_status launch_join_m(hape_join* h, const JoinArgs& a, bool mat, uint
     if (mat) return launch_join_t<KW, PRW, PSW, true, 2, 512>(h, a, ctas);
     return launch_join_t<KW, PRW, PSW, false, 2, 512>(h, a, ctas);
   }
-  // key|next nodes (one shared load per chain hop) for bag semantics, whose
-  // probes walk every chain to its end (C2 bag build+probe 1.023 -> 0.964 ms);
-  // a declared-unique build side stops at the first match, where the 8-byte
-  // node loads cost more bank conflicts than the hop saves (0.742 -> 1.181 ms).
-  // HAPE_JN_KN=0/1 forces the layout (A/B, tests)
-  static const int kn_env = env_int("HAPE_JN_KN", -1);
-  const bool kn = kn_env >= 0 ? kn_env != 0 : a.r_unique == 0;
-  if (kn) {
-    if (mat) return launch_join_t<KW, PRW, PSW, true, 0, 256, true>(h, a, ctas);
-    return launch_join_t<KW, PRW, PSW, false, 0, 256, true>(h, a, ctas);
+  // table layout (kernels.cuh JN_*): key|next nodes (one shared load per
+  // chain hop) for bag semantics, whose probes walk every chain to its end
+  // (C2 bag build+probe 1.023 -> 0.907 ms); a declared-unique build side
+  // stops at the first match, where the 8-byte node loads cost more bank
+  // conflicts than the hop saves (0.722 -> 1.020 ms).  HAPE_JN_LAY=0/1/2
+  // forces the layout (A/B, tests)
+  static const int lay_env = env_int("HAPE_JN_LAY", -1);
+  const int lay = lay_env >= 0 ? lay_env : (a.r_unique == 0 ? JN_KN : JN_AOS);
+  if (lay == JN_KN) {
+    if (mat) return launch_join_t<KW, PRW, PSW, true, 0, 256, JN_KN>(h, a, ctas);
+    return launch_join_t<KW, PRW, PSW, false, 0, 256, JN_KN>(h, a, ctas);
+  }
+  if (lay == JN_SK) {
+    if (mat) return launch_join_t<KW, PRW, PSW, true, 0, 256, JN_SK>(h, a, ctas);
+    return launch_join_t<KW, PRW, PSW, false, 0, 256, JN_SK>(h, a, ctas);
   }
   if (mat) return launch_join_t<KW, PRW, PSW, true, 0, 256>(h, a, ctas);
   return launch_join_t<KW, PRW, PSW, false, 0, 256>(h, a, ctas);

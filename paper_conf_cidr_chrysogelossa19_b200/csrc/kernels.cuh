@@ -1150,15 +1150,26 @@ __host__ __device__ constexpr size_t join_stile_bytes() {
 }
 // nrb R-chunk buffers, nsb staged S tiles of SU*256 tuples (SU = 0: S read
 // straight from HBM)
-// KN (key|next nodes): the build moves each R payload to pay[] and stores
-// the chain link in the tuple's payload field, so a chain hop is one shared
-// load of {key, next}; otherwise a u16 next[] array beside the tuples
-template <int KW, int PRW, int PSW, int SU = 0, int NC = 256, bool KN = false>
+// Table layouts (LAY):
+//   JN_AOS (0): chains over the landed AoS R tuples, a u16 next[] beside them;
+//   JN_KN  (1): key|next nodes -- the build moves each R payload to pay[] and
+//               stores the chain link in the tuple's payload field, so a chain
+//               hop is one shared load of {key, next};
+//   JN_SK  (2): the build also copies the keys to a dense keys[] array: a key
+//               load spreads over all 32 banks (a key inside 8-byte AoS tuples
+//               only reaches the 16 even ones); payloads stay in the tuples
+constexpr int JN_AOS = 0, JN_KN = 1, JN_SK = 2;
+template <int KW, int PRW>
+__host__ __device__ constexpr size_t join_link_bytes(uint32_t cap, int lay) {
+  return lay == JN_KN ? ((size_t)cap * PRW + 15) / 16 * 16
+                      : ((size_t)cap * 2 + 15) / 16 * 16 + (lay == JN_SK ? ((size_t)cap * KW + 15) / 16 * 16 : 0);
+}
+template <int KW, int PRW, int PSW, int SU = 0, int NC = 256, int LAY = JN_AOS>
 __host__ __device__ constexpr size_t join_smem_bytes(uint32_t cap, uint32_t slot_bits, uint32_t nrb = 2,
                                                      uint32_t nsb = 0) {
   return nrb * join_ring_bytes<KW, PRW>(cap)                               // R ring
          + (SU ? nsb * join_stile_bytes<KW, PSW, SU, NC>() : 0)           // S ring
-         + ((size_t)cap * (KN ? PRW : 2) + 15) / 16 * 16                   // pay[] / next[]
+         + join_link_bytes<KW, PRW>(cap, LAY)                              // next[] / pay[] / keys[]
          + (sizeof(JnHead) << slot_bits);                                  // heads[]
 }
 
@@ -1200,31 +1211,44 @@ struct JnAcc {
   unsigned long long cnt = 0, sr = 0, ss = 0, sx = 0;
 };
 
-template <int KW, int PRW, bool KN = false>
+template <int KW, int PRW, int LAY = JN_AOS>
 struct JnTable {
+  using K = typename UW<KW>::T;
   using V = typename UW<PRW>::T;
-  const Tup<KW, PRW>* r;    // R chunk (ring buffer); KN: {key, next} nodes
-  const void* link;         // next[] (u16), or KN: pay[] (the R payloads)
+  const Tup<KW, PRW>* r;    // R chunk (ring buffer); JN_KN: {key, next} nodes
+  const void* link;         // next[] (u16), or JN_KN: pay[] (the R payloads)
+  const K* keys;            // JN_SK: dense keys[]
   const JnHead* head;
   uint32_t sbits;
   bool dup;                 // the chunk holds some key twice (bag semantics path)
   uint32_t ep;              // stage epoch: a head is valid iff its high half == ep
-  // chain successor of e, whose tuple y = r[e] is already loaded
+  // does entry e hold key k?  (loads y = r[e] where the layout keeps the
+  // key in the tuple)
+  __device__ __forceinline__ bool hit(uint32_t e, K k, Tup<KW, PRW>& y) const {
+    if constexpr (LAY == JN_SK) return keys[e] == k;
+    else { y = r[e]; return y.k == k; }
+  }
+  // chain successor of e (y as loaded by hit(e))
   __device__ __forceinline__ uint32_t next_of(uint32_t e, const Tup<KW, PRW>& y) const {
-    if constexpr (KN) return (uint32_t)y.v;
+    if constexpr (LAY == JN_KN) return (uint32_t)y.v;
     else return static_cast<const uint16_t*>(link)[e];
   }
   __device__ __forceinline__ uint32_t next_at(uint32_t e) const {
-    if constexpr (KN) return (uint32_t)r[e].v;
+    if constexpr (LAY == JN_KN) return (uint32_t)r[e].v;
     else return static_cast<const uint16_t*>(link)[e];
   }
-  // R payload of e (y = r[e] already loaded)
+  __device__ __forceinline__ K key_at(uint32_t e) const {
+    if constexpr (LAY == JN_SK) return keys[e];
+    else return r[e].k;
+  }
+  // R payload of e (y as loaded by hit(e))
   __device__ __forceinline__ V pay_of(uint32_t e, const Tup<KW, PRW>& y) const {
-    if constexpr (KN) return static_cast<const V*>(link)[e];
+    if constexpr (LAY == JN_KN) return static_cast<const V*>(link)[e];
+    else if constexpr (LAY == JN_SK) return r[e].v;
     else return y.v;
   }
   __device__ __forceinline__ V pay_at(uint32_t e) const {
-    if constexpr (KN) return static_cast<const V*>(link)[e];
+    if constexpr (LAY == JN_KN) return static_cast<const V*>(link)[e];
     else return r[e].v;
   }
 };
@@ -1248,8 +1272,8 @@ __device__ __forceinline__ void jn_load_batch(const JoinArgs& a, uint32_t base, 
 }
 
 // Probe the U S tuples x[] (loaded by jn_load_batch for the same base).
-template <int KW, int PRW, int PSW, bool MAT, int U, int JN_CONSUMERS, bool KN>
-__device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, KN>& t, const JoinArgs& a, uint32_t base,
+template <int KW, int PRW, int PSW, bool MAT, int U, int JN_CONSUMERS, int LAY>
+__device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, LAY>& t, const JoinArgs& a, uint32_t base,
                                                uint32_t s_hi, const Tup<KW, PSW> (&x)[U], JnAcc& acc,
                                                uint32_t* s_wsum, unsigned long long* s_wbase) {
   using PR = typename UW<PRW>::S;
@@ -1276,10 +1300,15 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, KN>& t, co
       // load per visited tuple gives key and payload), aggregate once
       Tup<KW, PRW> y;
       while (e != JN_NIL) {
-        y = t.r[e];
-        if (y.k == x[u].k) break;
+        if (t.hit(e, x[u].k, y)) break;
         e = t.next_of(e, y);
       }
+      // reconverge before the aggregation body: without it the compiler
+      // ran the body of the KN / SK layouts once per group of lanes leaving
+      // the walk together (the 37-instruction body 2.7x per warp round: 1.03
+      // vs 0.75 ms); the AoS walk reconverges by itself and is faster
+      // without the explicit barrier (0.718 vs 0.750 ms)
+      if constexpr (LAY != JN_AOS) __syncwarp();
       if (e != JN_NIL) {
         const int64_t pr = (int64_t)(PR)t.pay_of(e, y), ps = (int64_t)(PS)x[u].v;
         if (MAT) m[u] = e;
@@ -1292,8 +1321,7 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, KN>& t, co
       while (true) {
         Tup<KW, PRW> y;
         while (e != JN_NIL) {
-          y = t.r[e];
-          if (y.k == x[u].k) break;
+          if (t.hit(e, x[u].k, y)) break;
           e = t.next_of(e, y);
         }
         const bool hit = e != JN_NIL;
@@ -1364,7 +1392,7 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, KN>& t, co
       if (!c[u]) continue;
       unsigned long long pos = wb + before[u] + incl[u] - c[u];
       for (uint32_t e = e0[u]; e != JN_NIL; e = t.next_at(e)) {
-        if (t.r[e].k == x[u].k) {
+        if (t.key_at(e) == x[u].k) {
           if (pos < a.out_cap) {
             static_cast<PR*>(a.out_r)[pos] = (PR)t.pay_at(e);
             static_cast<PS*>(a.out_s)[pos] = (PS)x[u].v;
@@ -1394,7 +1422,7 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, KN>& t, co
 // 544-thread CTA per SM, 36 % barrier stalls): C3 build+probe 15.3 vs 10.6 ms
 #define HAPE_JN_SR_MINB 2
 #endif
-template <int KW, int PRW, int PSW, bool MAT, int SU, int JN_CONSUMERS = 256, bool KN = false>
+template <int KW, int PRW, int PSW, bool MAT, int SU, int JN_CONSUMERS = 256, int LAY = JN_AOS>
 __global__ void __launch_bounds__(JN_CONSUMERS + 32,
                                   SU == 0 ? ((KW + PSW <= 8 && !MAT) ? HAPE_JN_MINB : 1) : HAPE_JN_SR_MINB)
 k_build_probe(JoinArgs a) {
@@ -1409,9 +1437,12 @@ k_build_probe(JoinArgs a) {
   const uint32_t NRB = a.nrb, NSB = SR ? a.nsb : 0u;
   unsigned char* ring = smem;                                           // [NRB][RB]
   unsigned char* sring = smem + NRB * RB;                               // [NSB][SB]
-  uint16_t* s_next = reinterpret_cast<uint16_t*>(sring + NSB * SB);               // !KN
-  typename UW<PRW>::T* s_pay = reinterpret_cast<typename UW<PRW>::T*>(sring + NSB * SB);  // KN
-  JnHead* s_head = reinterpret_cast<JnHead*>(sring + NSB * SB + ((size_t)a.cap * (KN ? PRW : 2) + 15) / 16 * 16);
+  constexpr bool KN = LAY == JN_KN;
+  using K = typename UW<KW>::T;
+  uint16_t* s_next = reinterpret_cast<uint16_t*>(sring + NSB * SB);               // JN_AOS / JN_SK
+  typename UW<PRW>::T* s_pay = reinterpret_cast<typename UW<PRW>::T*>(sring + NSB * SB);  // JN_KN
+  K* s_keys = reinterpret_cast<K*>(sring + NSB * SB + ((size_t)a.cap * 2 + 15) / 16 * 16);  // JN_SK
+  JnHead* s_head = reinterpret_cast<JnHead*>(sring + NSB * SB + join_link_bytes<KW, PRW>(a.cap, LAY));
   constexpr int MAXS = 8;
   __shared__ JnStage s_meta[2];
   __shared__ uint32_t s_soff[MAXS];
@@ -1523,8 +1554,12 @@ k_build_probe(JoinArgs a) {
             s_pay[i] = y.v;
             rw[i].v = (typename UW<PRW>::T)nx;
           }
-          // generic-proxy writes into a buffer the bulk-copy engine refills
-          asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
+        } else if constexpr (LAY == JN_SK) {
+          for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS) {
+            const K k = r[i].k;
+            s_keys[i] = k;
+            s_next[i] = (uint16_t)jn_head(atomicExch(&s_head[jn_slot<KW>(k, a.slot_bits)], (ep << 16) | i), ep);
+          }
         } else {
           for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
             s_next[i] = (uint16_t)jn_head(atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], (ep << 16) | i), ep);
@@ -1534,8 +1569,8 @@ k_build_probe(JoinArgs a) {
       // ---- probe (a12): stream the S slice.  Bag semantics walk every chain
       // to its end; a caller-declared unique build side (HAPE_FLAG_R_UNIQUE, a
       // primary key) stops at the first match.
-      const JnTable<KW, PRW, KN> tab{r, KN ? static_cast<const void*>(s_pay) : static_cast<const void*>(s_next),
-                                     s_head, a.slot_bits, a.r_unique == 0, ep};
+      const JnTable<KW, PRW, LAY> tab{r, KN ? static_cast<const void*>(s_pay) : static_cast<const void*>(s_next),
+                                      s_keys, s_head, a.slot_bits, a.r_unique == 0, ep};
       if constexpr (SR) {
         // staged S tiles: wait for the tile, copy this thread's tuples to
         // registers, release the tile (one arrival per warp), probe
@@ -1559,7 +1594,7 @@ k_build_probe(JoinArgs a) {
             consumer_sync<JN_CONSUMERS>();
             if (threadIdx.x == 0) mbar_arrive(&sempty[sb]);
           }
-          jn_probe_batch<KW, PRW, PSW, MAT, XU, JN_CONSUMERS, KN>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+          jn_probe_batch<KW, PRW, PSW, MAT, XU, JN_CONSUMERS, LAY>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
         }
       } else {
         // Full batches are software pipelined (PIPE): batch b+1 is loaded into
@@ -1574,7 +1609,7 @@ k_build_probe(JoinArgs a) {
           } else {
             jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, base, st.s_hi, x);
           }
-          jn_probe_batch<KW, PRW, PSW, MAT, JN_U, JN_CONSUMERS, KN>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+          jn_probe_batch<KW, PRW, PSW, MAT, JN_U, JN_CONSUMERS, LAY>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
           base += BATCH;
         }
         // ragged tail (< BATCH tuples, any JN_U): 4-, 2- and 1-wide batches
@@ -1584,21 +1619,25 @@ k_build_probe(JoinArgs a) {
           if (rem > 2 * JN_CONSUMERS) {
             Tup<KW, PSW> x[4];
             jn_load_batch<KW, PSW, 4, JN_CONSUMERS>(a, base, st.s_hi, x);
-            jn_probe_batch<KW, PRW, PSW, MAT, 4, JN_CONSUMERS, KN>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+            jn_probe_batch<KW, PRW, PSW, MAT, 4, JN_CONSUMERS, LAY>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
             base += 4 * JN_CONSUMERS;
           } else if (rem > JN_CONSUMERS) {
             Tup<KW, PSW> x[2];
             jn_load_batch<KW, PSW, 2, JN_CONSUMERS>(a, base, st.s_hi, x);
-            jn_probe_batch<KW, PRW, PSW, MAT, 2, JN_CONSUMERS, KN>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+            jn_probe_batch<KW, PRW, PSW, MAT, 2, JN_CONSUMERS, LAY>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
             base += 2 * JN_CONSUMERS;
           } else {
             Tup<KW, PSW> x[1];
             jn_load_batch<KW, PSW, 1, JN_CONSUMERS>(a, base, st.s_hi, x);
-            jn_probe_batch<KW, PRW, PSW, MAT, 1, JN_CONSUMERS, KN>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
+            jn_probe_batch<KW, PRW, PSW, MAT, 1, JN_CONSUMERS, LAY>(tab, a, base, st.s_hi, x, acc, s_wsum, s_wbase);
             base += JN_CONSUMERS;
           }
         }
       }
+      // KN: generic-proxy writes went into ring buffer bi, which the
+      // bulk-copy engine refills next (fenced here, after the probe: a fence
+      // right after the build also waited for the S batch loads in flight)
+      if constexpr (KN) asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
       consumer_sync<JN_CONSUMERS>();  // everyone is done with heads/next and ring buffer bi
       if (threadIdx.x == 0) mbar_arrive(&empty[bi]);
     }

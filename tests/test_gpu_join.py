@@ -422,8 +422,9 @@ def test_open_addressing_refill_cases(identity):
                                  dict(HAPE_JN_OA="1"), dict(HAPE_JN_SU="2"), dict(HAPE_JN_SU="0"),
                                  dict(HAPE_SC_AGG="1"), dict(HAPE_SC_AGG="2"),
                                  dict(HAPE_JN_EPOCH_PERIOD="1"), dict(HAPE_JN_EPOCH_PERIOD="3"),
-                                 dict(HAPE_JN_KN="1"), dict(HAPE_JN_KN="0"), dict(HAPE_JN_KN="1", HAPE_JN_SU="0"),
-                                 dict(HAPE_JN_KN="1", HAPE_JN_EPOCH_PERIOD="1")])
+                                 dict(HAPE_JN_LAY="1"), dict(HAPE_JN_LAY="0"), dict(HAPE_JN_LAY="2"),
+                                 dict(HAPE_JN_LAY="1", HAPE_JN_SU="0"), dict(HAPE_JN_LAY="2", HAPE_JN_SU="0"),
+                                 dict(HAPE_JN_LAY="1", HAPE_JN_EPOCH_PERIOD="1")])
 def test_alternative_kernel_forms_vs_oracle(env):
     # the retained alternatives, each read once per process (child process):
     # HAPE_JOINT=0 the per-pass totals + claiming scatters (the path of plans
@@ -431,8 +432,8 @@ def test_alternative_kernel_forms_vs_oracle(env):
     # HAPE_JN_OA=1 the open-addressing build+probe, HAPE_JN_SU the staged-S /
     # direct build+probe forms, HAPE_SC_AGG the warp-aggregated rankings,
     # HAPE_JN_EPOCH_PERIOD the chain-head epoch wrap (reset every 1 / 3 stages),
-    # HAPE_JN_KN the key|next node table of the direct build+probe (default
-    # for bag semantics only) forced on / off
+    # HAPE_JN_LAY the direct build+probe's table layouts forced (0 AoS
+    # tuples + next[], 1 key|next nodes -- the bag default, 2 dense keys[])
     import subprocess
     import sys
     import os
