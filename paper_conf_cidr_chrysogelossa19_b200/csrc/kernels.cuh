@@ -1508,6 +1508,20 @@ k_build_probe(JoinArgs a) {
             if (c_lo == r_lo && s_hi > s_lo && a.pf_bytes)
               bulk_prefetch_l2(sT + s_lo, min((size_t)(s_hi - s_lo) * sizeof(TS), (size_t)a.pf_bytes));
           }
+          // warm L2 with the next item's R chunk (and the head of its S
+          // slice): its bulk copy, issued once this stage releases the ring,
+          // then streams from L2 instead of HBM
+          if ((a.dbg & 8u) == 0 && c_lo == r_lo && it + gridDim.x < n_items) {
+            const uint2 nx = a.items[it + gridDim.x];
+            const uint32_t nr_lo = a.bR[nx.x], nr_hi = min(a.bR[nx.x + 1], nr_lo + a.cap);
+            if (nr_hi > nr_lo) bulk_prefetch_l2(rT + nr_lo, (size_t)(nr_hi - nr_lo) * sizeof(TR));
+            if (!SR && a.pf_bytes) {
+              const uint32_t ns_lo = a.bS[nx.x] + nx.y * a.slice;
+              const uint32_t ns_hi = min(a.bS[nx.x + 1], ns_lo + a.slice);
+              if (ns_hi > ns_lo)
+                bulk_prefetch_l2(sT + ns_lo, min((size_t)(ns_hi - ns_lo) * sizeof(TS), (size_t)a.pf_bytes));
+            }
+          }
         }
       }
       const uint32_t bi = stage % NRB, ph = (stage / NRB) & 1;
