@@ -563,6 +563,19 @@ def main():
                 # point of the plan, P723-724); frac = that transfer time / step
                 "pcie_roofline": {"bytes": h2d, "h2d_GB/s_measured": round(pcie_gbs, 1) if pcie_gbs else None,
                                   "frac": round((h2d / (pcie_gbs * 1e9) * 1000.0) / cp_ms, 3) if pcie_gbs else None},
+                # the plan's serial bound: a two-phase host partition completes
+                # every co-partition at the same moment, so no transfer can
+                # start before the host step ends (out-of-HBM: the device
+                # cannot stage pairs it cannot join yet); then every byte
+                # crosses PCIe once and the last pair's join follows its copy
+                "serial_bound": {
+                    "host_partition_ms": round(agg.get("host_part", 0), 3),
+                    "pcie_ms": round(h2d / (pcie_gbs * 1e9) * 1000.0, 3) if pcie_gbs else None,
+                    "last_pair_join_ms": round(dev / max(1, rc.n_partitions), 3),
+                    "frac": round((agg.get("host_part", 0) + h2d / (pcie_gbs * 1e9) * 1000.0
+                                   + dev / max(1, rc.n_partitions)) / cp_ms, 3) if pcie_gbs else None,
+                    "host_partition_GB/s": round(2 * h2d / (agg["host_part"] / 1000.0) / 1e9, 1)
+                    if agg.get("host_part") else None},
                 "same_result_as_radix": rc.as_tuple() == res.as_tuple()}
         del hk, ho
 

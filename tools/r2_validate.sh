@@ -11,7 +11,7 @@ for tool in memcheck racecheck synccheck; do
   echo "== compute-sanitizer --tool $tool --kernel-regex kns=hape python tools/sanitize_case.py" >> $S
   timeout 1200 compute-sanitizer --tool $tool --kernel-regex kns=hape python tools/sanitize_case.py 2>&1 | grep -E "SANITIZE|SUMMARY|Invalid|Race|error" | head -8 >> $S
 done
-for envv in HAPE_JN_SU=2 HAPE_JN_OA=1; do
+for envv in HAPE_JN_SU=2 HAPE_JN_OA=1 HAPE_JN_LAY=1 HAPE_JN_LAY=2; do
   echo "== $envv compute-sanitizer --tool memcheck" >> $S
   env $envv timeout 900 compute-sanitizer --tool memcheck --kernel-regex kns=hape python tools/sanitize_case.py 2>&1 | grep -E "SANITIZE|SUMMARY|Invalid|error" | head -8 >> $S
 done
