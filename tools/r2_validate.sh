@@ -6,7 +6,11 @@ TAG=${1:-r2v}
 mkdir -p gpurun_out
 python -c "import __graft_entry__ as g; g.build(); g.smoke()" 2>&1 | tail -1
 timeout 1800 python -m pytest tests -m gpu -q 2>&1 | tail -4 | tee gpurun_out/tests_$TAG.log
+# compute-sanitizer: closed on this GPU pool from round 2 on ("runs under it
+# have left GPUs needing a reset"); the last sanitizer evidence is
+# profiles/r2/sanitizers_r2w.txt.  SANITIZE=1 runs it where it is allowed.
 S=gpurun_out/sanitizers_$TAG.txt; : > $S
+if [ -n "$SANITIZE" ]; then
 for tool in memcheck racecheck synccheck; do
   echo "== compute-sanitizer --tool $tool --kernel-regex kns=hape python tools/sanitize_case.py" >> $S
   timeout 1200 compute-sanitizer --tool $tool --kernel-regex kns=hape python tools/sanitize_case.py 2>&1 | grep -E "SANITIZE|SUMMARY|Invalid|Race|error" | head -8 >> $S
@@ -14,6 +18,12 @@ done
 for envv in HAPE_JN_SU=2 HAPE_JN_OA=1 HAPE_JN_LAY=1 HAPE_JN_LAY=2; do
   echo "== $envv compute-sanitizer --tool memcheck" >> $S
   env $envv timeout 900 compute-sanitizer --tool memcheck --kernel-regex kns=hape python tools/sanitize_case.py 2>&1 | grep -E "SANITIZE|SUMMARY|Invalid|error" | head -8 >> $S
+done
+fi
+# the sanitizer case without the sanitizer (every kernel family, bag and unique layouts)
+for envv in HAPE_JN_LAY=-1 HAPE_JN_LAY=0 HAPE_JN_LAY=1 HAPE_JN_LAY=2 HAPE_JN_SU=2; do
+  echo "== $envv python tools/sanitize_case.py" >> $S
+  env $envv timeout 600 python tools/sanitize_case.py 2>&1 | grep -E "SANITIZE|Error|error" | head -3 >> $S
 done
 cat $S
 timeout 900 python bench.py > gpurun_out/bench_default_$TAG.json 2> gpurun_out/bench_default_$TAG.err
