@@ -1148,6 +1148,9 @@ k_worklist(const uint32_t* __restrict__ bR, const uint32_t* __restrict__ bS, uin
 #define HAPE_JN_U 2
 #endif
 constexpr int JN_U = HAPE_JN_U;
+#ifndef HAPE_JN_PTAIL
+#define HAPE_JN_PTAIL 1
+#endif
 
 #ifndef HAPE_JN_REL_MODE
 #define HAPE_JN_REL_MODE 1
@@ -1225,6 +1228,14 @@ struct JnStage {
   uint32_t s_lo, s_hi;
 };
 
+// slot and mbarrier phase of the seq-th use of an n-deep ring (n is 1 or 2
+// on the hot paths: no integer division per stage)
+__device__ __forceinline__ void ring_pos(uint32_t seq, uint32_t n, uint32_t& slot, uint32_t& phase) {
+  if (n == 1) { slot = 0; phase = seq & 1u; }
+  else if (n == 2) { slot = seq & 1u; phase = (seq >> 1) & 1u; }
+  else { slot = seq % n; phase = (seq / n) & 1u; }
+}
+
 template <int NC>
 __device__ __forceinline__ void consumer_sync() {
   asm volatile("bar.sync 1, %0;" ::"n"(NC) : "memory");
@@ -1287,7 +1298,10 @@ struct JnTable {
 // earlier stage (other epoch) reads as an empty chain, so the heads are never
 // reset between stages
 __device__ __forceinline__ uint32_t jn_head(JnHead hv, uint32_t ep) {
-  return (hv >> 16) == ep ? (hv & 0xFFFFu) : JN_NIL;
+  // heads of earlier epochs (and the zeroed epoch 0) are smaller than
+  // ep << 16, so the difference wraps above 0xFFFF: one subtract and one
+  // unsigned min instead of a shift, compare, mask and select
+  return min(hv - (ep << 16), 0xFFFFu);
 }
 
 // Load U S tuples per consumer thread: j = base + u*256 + tid.  (Two
@@ -1515,7 +1529,8 @@ k_build_probe(JoinArgs a) {
         const uint32_t s_lo = a.bS[q] + item.y * a.slice;
         const uint32_t s_hi = min(a.bS[q + 1], s_lo + a.slice);
         for (uint32_t c_lo = r_lo; c_lo < r_hi; c_lo += a.cap, stage++) {
-          const uint32_t bi = stage % NRB, ph = (stage / NRB) & 1;
+          uint32_t bi, ph;
+      ring_pos(stage, NRB, bi, ph);
           mbar_wait_backoff(&empty[bi], ph ^ 1);
           const uint32_t nr = min(a.cap, r_hi - c_lo);
           const uintptr_t ra = reinterpret_cast<uintptr_t>(rT + c_lo);
@@ -1526,7 +1541,8 @@ k_build_probe(JoinArgs a) {
           if constexpr (SR) {
             // the stage's S slice, tile by tile, through the S ring
             for (uint32_t t0 = s_lo; t0 < s_hi; t0 += JN_STILE, sseq++) {
-              const uint32_t sb = sseq % NSB, sph = (sseq / NSB) & 1;
+              uint32_t sb, sph;
+              ring_pos(sseq, NSB, sb, sph);
               mbar_wait_backoff(&sempty[sb], sph ^ 1);
               const uint32_t n = min(JN_STILE, s_hi - t0);
               const uintptr_t sa = reinterpret_cast<uintptr_t>(sT + t0);
@@ -1556,7 +1572,8 @@ k_build_probe(JoinArgs a) {
           }
         }
       }
-      const uint32_t bi = stage % NRB, ph = (stage / NRB) & 1;
+      uint32_t bi, ph;
+      ring_pos(stage, NRB, bi, ph);
       mbar_wait_backoff(&empty[bi], ph ^ 1);
       s_meta[bi].nr = JN_STOP;
       mbar_arrive(&full[bi]);
@@ -1565,7 +1582,8 @@ k_build_probe(JoinArgs a) {
     // ------------------------------ consumer warps -----------------------------
     uint32_t sseq = 0, ep = 0;
     for (uint32_t stage = 0;; stage++) {
-      const uint32_t bi = stage % NRB, ph = (stage / NRB) & 1;
+      uint32_t bi, ph;
+      ring_pos(stage, NRB, bi, ph);
       // stage epoch (1..ep_period, ep_period <= 65535): heads of other
       // epochs read as empty chains, so the table needs no reset; every
       // ep_period stages the heads are zeroed (epoch 0 is never used) -- the
@@ -1589,7 +1607,10 @@ k_build_probe(JoinArgs a) {
       // slower for C3)
       constexpr bool PIPE = !MAT && !SR;
       Tup<KW, PSW> xs[JN_U];
-      if (PIPE && st.s_lo + BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, st.s_lo, st.s_hi, xs);
+      // (PTAIL: the ragged last batch is pipelined too, its loads predicated)
+      constexpr bool PTAIL = PIPE && HAPE_JN_PTAIL;
+      if (PIPE && (PTAIL ? st.s_lo < st.s_hi : st.s_lo + BATCH <= st.s_hi))
+        jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, st.s_lo, st.s_hi, xs);
       if (!(a.dbg & 4u)) {
         if constexpr (KN) {
           // the payload moves to pay[i], the link takes its place in the node
@@ -1621,7 +1642,8 @@ k_build_probe(JoinArgs a) {
         // staged S tiles: wait for the tile, copy this thread's tuples to
         // registers, release the tile (one arrival per warp), probe
         for (uint32_t base = st.s_lo; base < st.s_hi; base += JN_STILE, sseq++) {
-          const uint32_t sb = sseq % NSB, sph = (sseq / NSB) & 1;
+          uint32_t sb, sph;
+              ring_pos(sseq, NSB, sb, sph);
           mbar_wait(&sfull[sb], sph);
           const TS* tile = reinterpret_cast<const TS*>(sring + sb * SB + s_soff[sb]);
           const uint32_t n = min(JN_STILE, st.s_hi - base);
@@ -1646,12 +1668,27 @@ k_build_probe(JoinArgs a) {
         // Full batches are software pipelined (PIPE): batch b+1 is loaded into
         // registers while b is probed.
         uint32_t base = st.s_lo;
-        while (base + BATCH <= st.s_hi) {
+        if constexpr (PTAIL) {
+          // two register sets alternate (unrolled by two): no copy of the
+          // prefetched batch into the probed one
+          Tup<KW, PSW> xt[JN_U];
+          while (base < st.s_hi) {
+            if (base + BATCH < st.s_hi) jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, base + BATCH, st.s_hi, xt);
+            jn_probe_batch<KW, PRW, PSW, MAT, JN_U, JN_CONSUMERS, LAY>(tab, a, base, st.s_hi, xs, acc, s_wsum, s_wbase);
+            base += BATCH;
+            if (base >= st.s_hi) break;
+            if (base + BATCH < st.s_hi) jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, base + BATCH, st.s_hi, xs);
+            jn_probe_batch<KW, PRW, PSW, MAT, JN_U, JN_CONSUMERS, LAY>(tab, a, base, st.s_hi, xt, acc, s_wsum, s_wbase);
+            base += BATCH;
+          }
+        }
+        while (!PTAIL && base + BATCH <= st.s_hi) {
           Tup<KW, PSW> x[JN_U];
           if constexpr (PIPE) {
 #pragma unroll
             for (int u = 0; u < JN_U; u++) x[u] = xs[u];
-            if (base + 2 * BATCH <= st.s_hi) jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, base + BATCH, st.s_hi, xs);
+            if (PTAIL ? base + BATCH < st.s_hi : base + 2 * BATCH <= st.s_hi)
+              jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, base + BATCH, st.s_hi, xs);
           } else {
             jn_load_batch<KW, PSW, JN_U, JN_CONSUMERS>(a, base, st.s_hi, x);
           }
@@ -1659,8 +1696,9 @@ k_build_probe(JoinArgs a) {
           base += BATCH;
         }
         // ragged tail (< BATCH tuples, any JN_U): 4-, 2- and 1-wide batches
-        // until the slice is exhausted (rem is uniform over the consumers)
-        while (st.s_hi > base) {
+        // until the slice is exhausted (rem is uniform over the consumers);
+        // PTAIL forms have none left
+        while (!PTAIL && st.s_hi > base) {
           const uint32_t rem = st.s_hi - base;
           if (rem > 2 * JN_CONSUMERS) {
             Tup<KW, PSW> x[4];
