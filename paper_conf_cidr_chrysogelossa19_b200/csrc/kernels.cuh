@@ -1144,8 +1144,11 @@ k_worklist(const uint32_t* __restrict__ bR, const uint32_t* __restrict__ bS, uin
 // --------------------------------------------------------------------------
 // consumer threads per build+probe CTA: a template parameter (JN_CONSUMERS,
 // 256 or 512) of the kernel; one producer warp on top
+// S tuples per consumer thread per batch of the direct form (C2 build+probe
+// with the pipelined tail: U = 1 / 2 / 3 / 4 -> 0.692 / 0.649 / 0.640 /
+// 0.654 ms; C4 10.05 -> 9.92, C5 3.89 -> 3.80 ms at 3)
 #ifndef HAPE_JN_U
-#define HAPE_JN_U 2
+#define HAPE_JN_U 3
 #endif
 constexpr int JN_U = HAPE_JN_U;
 #ifndef HAPE_JN_PTAIL
