@@ -269,13 +269,30 @@ __device__ __forceinline__ void mbar_expect_tx(uint64_t* bar, uint32_t bytes) {
 __device__ __forceinline__ void mbar_arrive(uint64_t* bar) {
   asm volatile("mbarrier.arrive.shared::cta.b64 _, [%0];" ::"r"(smem_u32(bar)) : "memory");
 }
+#ifndef HAPE_MBAR_SUSPEND
+#define HAPE_MBAR_SUSPEND 0
+#endif
 __device__ __forceinline__ void mbar_wait(uint64_t* bar, uint32_t phase) {
+#if HAPE_MBAR_SUSPEND
+  // suspend inside try_wait (time-limit hint) instead of re-issuing it: a
+  // waiting warp does not take issue slots from the warps that have work
+  uint32_t ok = 0;
+  while (true) {
+    asm volatile(
+        "{\n .reg .pred p;\n mbarrier.try_wait.parity.shared::cta.b64 p, [%1], %2, %3;\n selp.u32 %0, 1, 0, p;\n}\n"
+        : "=r"(ok)
+        : "r"(smem_u32(bar)), "r"(phase), "r"(HAPE_MBAR_SUSPEND)
+        : "memory");
+    if (ok) return;
+  }
+#else
   asm volatile(
       "{\n .reg .pred p;\n WAIT_%=:\n"
       " mbarrier.try_wait.parity.shared::cta.b64 p, [%0], %1;\n"
       " @!p bra WAIT_%=;\n}\n" ::"r"(smem_u32(bar)),
       "r"(phase)
       : "memory");
+#endif
 }
 // producer-side wait: the thread is suspended inside try_wait (time-limit
 // hint) instead of polling, so a warp that is far ahead does not steal issue
