@@ -1648,6 +1648,8 @@ k_build_probe(JoinArgs a) {
             s_next[i] = (uint16_t)jn_head(atomicExch(&s_head[jn_slot<KW>(k, a.slot_bits)], (ep << 16) | i), ep);
           }
         } else {
+          // (2 / 4 inserts per thread in flight measured 0.634 / 0.642 vs
+          // 0.638 ms: the exchanges are not the stage's critical path)
           for (uint32_t i = threadIdx.x; i < st.nr; i += JN_CONSUMERS)
             s_next[i] = (uint16_t)jn_head(atomicExch(&s_head[jn_slot<KW>(r[i].k, a.slot_bits)], (ep << 16) | i), ep);
         }
