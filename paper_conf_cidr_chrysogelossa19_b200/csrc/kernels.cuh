@@ -1173,13 +1173,16 @@ constexpr int JN_U = HAPE_JN_U;
 #endif
 
 #ifndef HAPE_JN_REL_MODE
-#define HAPE_JN_REL_MODE 1
+#define HAPE_JN_REL_MODE 0
 #endif
-// SR tile release after the consumers' copy to registers: 1 = one consumer
-// barrier, then one arrival (C3 build+probe 10.76 ms; racecheck-clean);
-// 0 = per-warp __syncwarp + lane-0 arrival (10.56 ms; correct by the PTX
-// model's cumulativity, but racecheck cannot see the ordering).  Releasing at
-// the materialising probe's claim barrier instead measured 14.4 ms (the refill
+// SR tile release after the consumers' copy to registers: 0 = per-warp
+// __syncwarp + lane-0 arrival on the tile's empty barrier (16 arrivals: the
+// producer/consumer pattern of TMA pipelines -- the warp's reads are ordered
+// before the release arrive, the producer's acquire wait before its refill;
+// C3 build+probe 10.13-10.22 -> 9.84-9.88 ms, round 2 default); 1 = one
+// consumer barrier, then one arrival (the form racecheck could verify, the
+// default while compute-sanitizer ran on this pool).  Releasing at the
+// materialising probe's claim barrier instead measured 14.4 ms (the refill
 // starts a whole probe later), and a runtime switch between the forms slowed
 // every form to ~14 ms (a barrier under a runtime branch), so the form is a
 // compile-time choice.
