@@ -690,6 +690,15 @@ static hape_status launch_join_m(hape_join* h, const JoinArgs& a, bool mat, uint
     return launch_join_t<KW, PRW, PSW, false, 0, 256, JN_SK>(h, a, ctas);
   }
   if (mat) return launch_join_t<KW, PRW, PSW, true, 0, 256>(h, a, ctas);
+  // large co-partitions (R chunks beyond ~3 K tuples: 16-bit plans over
+  // 2^28-tuple relations, C4's share at N = 8) run 512 consumer threads at 2
+  // CTAs per SM with a 2^13-slot table, where the 256-thread form drops to 3
+  // CTAs per SM at load factor 1 (C4/8 build+probe 1.466 -> 1.215 ms, 0.45 ->
+  // 0.54 of HBM); 2 K-tuple co-partitions stay on 256 (C2 0.643 vs 0.664 ms).
+  // HAPE_JN_NC=256/512 forces the shape (A/B)
+  static const int nc_env = env_int("HAPE_JN_NC", 0);
+  if (KW + PSW <= 8 && (nc_env == 512 || (nc_env == 0 && a.cap > 3072)))
+    return launch_join_t<KW, PRW, PSW, false, 0, 512>(h, a, ctas);
   return launch_join_t<KW, PRW, PSW, false, 0, 256>(h, a, ctas);
 }
 

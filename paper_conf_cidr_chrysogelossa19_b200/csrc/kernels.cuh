@@ -1496,7 +1496,8 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, LAY>& t, c
 #endif
 template <int KW, int PRW, int PSW, bool MAT, int SU, int JN_CONSUMERS = 256, int LAY = JN_AOS>
 __global__ void __launch_bounds__(JN_CONSUMERS + 32,
-                                  SU == 0 ? ((KW + PSW <= 8 && !MAT) ? HAPE_JN_MINB : 1) : HAPE_JN_SR_MINB)
+                                  SU == 0 ? ((KW + PSW <= 8 && !MAT) ? (JN_CONSUMERS == 256 ? HAPE_JN_MINB : 2) : 1)
+                                          : HAPE_JN_SR_MINB)
 k_build_probe(JoinArgs a) {
   constexpr int JN_THREADS = JN_CONSUMERS + 32;
   constexpr bool SR = SU > 0;

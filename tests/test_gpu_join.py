@@ -130,10 +130,13 @@ def test_c1_full_with_pairs_vs_oracle():
 @pytest.mark.parametrize("passes,bits", [(1, (0, 0)), (1, (4, 0)), (1, (11, 0)), (2, (3, 5)),
                                          (2, (8, 8)), (2, (12, 2)), (2, (6, 12)), (2, (10, 10)),
                                          (2, (12, 12)), (1, (12, 0))])
-def test_metamorphic_plans_identical(passes, bits):
+@pytest.mark.parametrize("uq", [False, True])
+def test_metamorphic_plans_identical(passes, bits, uq):
+    # uq: the declared-unique probe (large co-partitions of the coarse plans
+    # take the 512-consumer shape and R-chunking there)
     wl = datagen.make("c2", n_r=1 << 20, n_s=(1 << 20) + 3)
     ref = provenance.expected_from_workload(wl)
-    j = joiner(torch.int32, radix_passes=passes, radix_bits=bits)
+    j = joiner(torch.int32, radix_passes=passes, radix_bits=bits, r_unique=uq)
     res = j.join(cuda(wl.R.key), cuda(wl.R.payload), cuda(wl.S.key), cuda(wl.S.payload))
     check(res, ref)
     assert res.passes == passes
@@ -424,7 +427,8 @@ def test_open_addressing_refill_cases(identity):
                                  dict(HAPE_JN_EPOCH_PERIOD="1"), dict(HAPE_JN_EPOCH_PERIOD="3"),
                                  dict(HAPE_JN_LAY="1"), dict(HAPE_JN_LAY="0"), dict(HAPE_JN_LAY="2"),
                                  dict(HAPE_JN_LAY="1", HAPE_JN_SU="0"), dict(HAPE_JN_LAY="2", HAPE_JN_SU="0"),
-                                 dict(HAPE_JN_LAY="1", HAPE_JN_EPOCH_PERIOD="1")])
+                                 dict(HAPE_JN_LAY="1", HAPE_JN_EPOCH_PERIOD="1"),
+                                 dict(HAPE_JN_NC="512"), dict(HAPE_JN_NC="256")])
 def test_alternative_kernel_forms_vs_oracle(env):
     # the retained alternatives, each read once per process (child process):
     # HAPE_JOINT=0 the per-pass totals + claiming scatters (the path of plans
@@ -433,7 +437,8 @@ def test_alternative_kernel_forms_vs_oracle(env):
     # direct build+probe forms, HAPE_SC_AGG the warp-aggregated rankings,
     # HAPE_JN_EPOCH_PERIOD the chain-head epoch wrap (reset every 1 / 3 stages),
     # HAPE_JN_LAY the direct build+probe's table layouts forced (0 AoS
-    # tuples + next[], 1 key|next nodes -- the bag default, 2 dense keys[])
+    # tuples + next[], 1 key|next nodes -- the bag default, 2 dense keys[]),
+    # HAPE_JN_NC the unique direct form's 512- / 256-consumer shapes
     import subprocess
     import sys
     import os
