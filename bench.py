@@ -477,6 +477,31 @@ def main():
             if fused else "NCCL send/recv of a device-partitioned send buffer",
             "bound": "nvlink 900 GB/s/dir per GPU (remote part); HBM 2t B/tuple (read + write)"}
         roofline["exchange_path"] = res.exchange_path
+        if world > 1:
+            # the NVLink reference the exchange stage is read against (SURVEY
+            # §8.d.3): one NCCL all-to-all of the same bytes per rank, CUDA
+            # events on this stream, max over ranks
+            try:
+                buf = torch.empty(xb // 4 // world * world, dtype=torch.int32, device="cuda")
+                out = torch.empty_like(buf)
+                for _ in range(2):
+                    dist.all_to_all_single(out, buf)
+                barrier()
+                a0, a1 = torch.cuda.Event(enable_timing=True), torch.cuda.Event(enable_timing=True)
+                a0.record(stream)
+                for _ in range(3):
+                    dist.all_to_all_single(out, buf)
+                a1.record(stream)
+                barrier()
+                a_ms = max_over_ranks(a0.elapsed_time(a1) / 3)
+                nb = buf.numel() * 4
+                roofline["stages"]["exchange"]["nccl_all_to_all_reference"] = {
+                    "bytes_per_rank": nb, "ms": round(a_ms, 4),
+                    "algbw_GB/s": round(nb / (a_ms / 1000.0) / 1e9, 1),
+                    "busbw_GB/s": round(nb * (world - 1) / world / (a_ms / 1000.0) / 1e9, 1)}
+                del buf, out
+            except Exception as ex:  # never lose the line to the reference measurement
+                roofline["stages"]["exchange"]["nccl_all_to_all_reference"] = {"error": repr(ex)[:200]}
 
     # ---- end to end through the same C ABI call with pinned host buffers
     e2e = None
