@@ -289,10 +289,16 @@ struct Src {
 
 static size_t tup_bytes(int kw, int pw) { return (kw + pw) <= 8 ? 8 : 16; }
 
+// Workspace (AoS) tuples carry h(k) in their key field (kernels.cuh
+// HAPE_STORE_H): passes over them take buckets from it directly (IDENT)
+static bool ident_for(const hape_join* h, bool aos) {
+  return (HAPE_STORE_H && aos) || h->cfg.part_fn == HAPE_PART_IDENTITY;
+}
+
 template <int KW, int PW, bool AOS>
 static void hist_t(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* hist, uint32_t* rowsum) {
   const unsigned grid = m.nseg * m.cps;
-  if (h->cfg.part_fn == HAPE_PART_IDENTITY)
+  if (ident_for(h, AOS))
     k_hist<KW, PW, AOS, true><<<grid, HIST_THREADS, (size_t)P * 4, h->stream>>>(s.in, m, bf, P, hist, rowsum);
   else
     k_hist<KW, PW, AOS, false><<<grid, HIST_THREADS, (size_t)P * 4, h->stream>>>(s.in, m, bf, P, hist, rowsum);
@@ -396,7 +402,7 @@ static hape_status hist_joint_t(hape_join* h, const Src& s, SegMap m, BitField b
 template <int KW, int PW, bool AOS>
 static hape_status hist_joint_i(hape_join* h, const Src& s, SegMap m, BitField bf1, BitField bf2, uint32_t P1,
                                 uint32_t P2, uint32_t* rowsum, uint16_t* part, uint32_t* ovf) {
-  if (h->cfg.part_fn == HAPE_PART_IDENTITY)
+  if (ident_for(h, AOS))
     return hist_joint_t<KW, PW, AOS, true>(h, s, m, bf1, bf2, P1, P2, rowsum, part, ovf);
   return hist_joint_t<KW, PW, AOS, false>(h, s, m, bf1, bf2, P1, P2, rowsum, part, ovf);
 }
@@ -468,7 +474,7 @@ static hape_status scatter_t(hape_join* h, const Src& s, SegMap m, BitField bf, 
 template <int KW, int PW, bool AOS, class C>
 static hape_status scatter_linked_c(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, void* out,
                                     const LinkMap& lk) {
-  if (h->cfg.part_fn == HAPE_PART_IDENTITY)
+  if (ident_for(h, AOS))
     return scatter_t<KW, PW, AOS, C, true, true, true>(h, s, m, bf, P, lk.cnt, out, &lk);
   return scatter_t<KW, PW, AOS, C, false, true, true>(h, s, m, bf, P, lk.cnt, out, &lk);
 }
@@ -541,10 +547,10 @@ template <int KW, int PW, bool AOS>
 static hape_status scatter_v(hape_join* h, const Src& s, SegMap m, BitField bf, uint32_t P, uint32_t* offs,
                              void* out, bool claim) {
   if (claim) {
-    if (h->cfg.part_fn == HAPE_PART_IDENTITY) return scatter_i<KW, PW, AOS, true, true>(h, s, m, bf, P, offs, out);
+    if (ident_for(h, AOS)) return scatter_i<KW, PW, AOS, true, true>(h, s, m, bf, P, offs, out);
     return scatter_i<KW, PW, AOS, false, true>(h, s, m, bf, P, offs, out);
   }
-  if (h->cfg.part_fn == HAPE_PART_IDENTITY) return scatter_i<KW, PW, AOS, true, false>(h, s, m, bf, P, offs, out);
+  if (ident_for(h, AOS)) return scatter_i<KW, PW, AOS, true, false>(h, s, m, bf, P, offs, out);
   return scatter_i<KW, PW, AOS, false, false>(h, s, m, bf, P, offs, out);
 }
 
@@ -742,7 +748,7 @@ static hape_status launch_oa_m(hape_join* h, const JoinArgs& a, uint32_t* ctas) 
 
 template <int KW, int PRW, int PSW>
 static hape_status launch_oa_w(hape_join* h, const JoinArgs& a, bool mat, uint32_t* ctas) {
-  const bool ident = h->cfg.part_fn == HAPE_PART_IDENTITY;
+  const bool ident = ident_for(h, true);  // the workspace tuples' key field holds h(k)
   if (mat) return ident ? launch_oa_m<KW, PRW, PSW, true, true>(h, a, ctas)
                         : launch_oa_m<KW, PRW, PSW, true, false>(h, a, ctas);
   return ident ? launch_oa_m<KW, PRW, PSW, false, true>(h, a, ctas)
@@ -774,10 +780,12 @@ static hape_status launch_join(hape_join* h, int kw, int prw, int psw, const Joi
 static hape_status launch_unpack(hape_join* h, int kw, int pw, const void* t, uint32_t n, void* k, void* p) {
   if (!n) return HAPE_OK;
   const unsigned grid = std::min<unsigned>((n + 255) / 256, 4096);
-  if (kw == 4 && pw == 4) k_unpack<4, 4><<<grid, 256, 0, h->stream>>>((const Tup<4, 4>*)t, n, (uint32_t*)k, (uint32_t*)p);
-  else if (kw == 4) k_unpack<4, 8><<<grid, 256, 0, h->stream>>>((const Tup<4, 8>*)t, n, (uint32_t*)k, (uint64_t*)p);
-  else if (pw == 4) k_unpack<8, 4><<<grid, 256, 0, h->stream>>>((const Tup<8, 4>*)t, n, (uint64_t*)k, (uint32_t*)p);
-  else k_unpack<8, 8><<<grid, 256, 0, h->stream>>>((const Tup<8, 8>*)t, n, (uint64_t*)k, (uint64_t*)p);
+  // workspace tuples hold h(k): hand the key back (HAPE_STORE_H)
+  const uint32_t um = (HAPE_STORE_H && h->cfg.part_fn == HAPE_PART_HASH) ? 1u : 0u;
+  if (kw == 4 && pw == 4) k_unpack<4, 4><<<grid, 256, 0, h->stream>>>((const Tup<4, 4>*)t, n, (uint32_t*)k, (uint32_t*)p, um);
+  else if (kw == 4) k_unpack<4, 8><<<grid, 256, 0, h->stream>>>((const Tup<4, 8>*)t, n, (uint32_t*)k, (uint64_t*)p, um);
+  else if (pw == 4) k_unpack<8, 4><<<grid, 256, 0, h->stream>>>((const Tup<8, 4>*)t, n, (uint64_t*)k, (uint32_t*)p, um);
+  else k_unpack<8, 8><<<grid, 256, 0, h->stream>>>((const Tup<8, 8>*)t, n, (uint64_t*)k, (uint64_t*)p, um);
   CK_LAUNCH(h);
   return HAPE_OK;
 }

@@ -49,6 +49,21 @@ __device__ __forceinline__ uint64_t fmix64(uint64_t x) {
   return x;
 }
 
+// inverses of the two mixers (debug entry points only: they hand the
+// workspace's h(k) back to the caller as the key k)
+__device__ __forceinline__ uint32_t fmix32_inv(uint32_t h) {
+  h ^= h >> 16; h *= 0x7ed1b41du;
+  h ^= (h >> 13) ^ (h >> 26); h *= 0xa5cb9243u;
+  h ^= h >> 16;
+  return h;
+}
+__device__ __forceinline__ uint64_t fmix64_inv(uint64_t x) {
+  x ^= (x >> 31) ^ (x >> 62); x *= 0x319642b2d24d8ec3ull;
+  x ^= (x >> 27) ^ (x >> 54); x *= 0x96de1b173f119089ull;
+  x ^= (x >> 30) ^ (x >> 60);
+  return x;
+}
+
 // h(k): bijective mixer of the key bit pattern, or identity (P802-804)
 // (IDENT is a template parameter: the per-tuple paths carry no branch on it)
 template <int KW, bool IDENT>
@@ -756,6 +771,14 @@ k_scan(uint32_t* __restrict__ hist, const uint32_t* __restrict__ rowsum, SegMap 
 // or both at the end), so L2 merges it instead of evicting a half-written
 // sector and paying a DRAM read-modify-write.
 // --------------------------------------------------------------------------
+// The first scatter over the caller's SoA columns stores h(k) in the
+// workspace tuples' key field, so every later pass (and the hist / join
+// kernels over AoS workspace tuples) reads its buckets straight from it;
+// hape.cu launches those with IDENT = true.  0: keys stay raw (A/B only --
+// the host side must then launch AoS passes with the configured function).
+#ifndef HAPE_STORE_H
+#define HAPE_STORE_H 1
+#endif
 template <int NT_, int ITEMS_, int STAGES_, int MINB_ = 1024 / NT_, bool DST_ = false>
 struct ScCfg {
   static constexpr int NT = NT_, ITEMS = ITEMS_, STAGES = STAGES_, T = NT_ * ITEMS_, MINB = MINB_;
@@ -841,6 +864,8 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
   using Tp = Tup<KW, PW>;
   using L = ScLayout<KW, PW, AOS, C>;
   constexpr int NT = C::NT, T = C::T, ITEMS = C::ITEMS, STAGES = C::STAGES;
+  // SoA caller columns hashed here for the last time (HAPE_STORE_H)
+  constexpr bool STORE_H = HAPE_STORE_H && !AOS && !IDENT;
   extern __shared__ __align__(128) unsigned char smem[];
   unsigned char* raw = smem;                                            // [STAGES][RAW]
   const uint32_t P4 = (P + 3) & ~3u;                  // keep the arrays below 16-byte aligned
@@ -903,6 +928,14 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
     };
     mbar_wait(&bar[s], ph);
     // phase 1: bucket + rank (shared-memory atomic claim); tuples -> registers
+    // (STORE_H: the tuple keeps h(k) in its key field from here on -- h is a
+    // bijection, so later passes take their buckets from the stored value and
+    // the join compares h(k) for k; keys never leave the workspace)
+    auto hb = [&](Tp& t) -> uint32_t {
+      const uint64_t hv = part_hash<KW, IDENT>(t.k);
+      if constexpr (STORE_H) t.k = (K)hv;
+      return bucket_of(hv, bf);
+    };
     Tp x[ITEMS];
     uint32_t br[ITEMS];
     const bool full = tn == (uint32_t)T;
@@ -935,19 +968,19 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
       if (agg == 1) {
 #pragma unroll
         for (int u = 0; u < ITEMS; u++) {
-          const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
+          const uint32_t b = hb(x[u]);
           br[u] = (b << 16) | rank_agg(b, 0xffffffffu);
         }
       } else if (agg == 2) {
 #pragma unroll
         for (int u = 0; u < ITEMS; u++) {
-          const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
+          const uint32_t b = hb(x[u]);
           br[u] = (b << 16) | rank_hot(b);
         }
       } else {
 #pragma unroll
         for (int u = 0; u < ITEMS; u++) {
-          const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
+          const uint32_t b = hb(x[u]);
           br[u] = (b << 16) | atomicAdd(&s_cnt[b], 1u);
         }
       }
@@ -958,7 +991,7 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
         const uint32_t vm = __ballot_sync(0xffffffffu, i < tn);
         if (i < tn) {
           x[u] = load(i);
-          const uint32_t b = bucket_of(part_hash<KW, IDENT>(x[u].k), bf);
+          const uint32_t b = hb(x[u]);
           br[u] = (b << 16) | (agg == 1 ? rank_agg(b, vm) : atomicAdd(&s_cnt[b], 1u));
         }
       }
@@ -1074,15 +1107,15 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
       else if constexpr (LINKED) {
         // one 8-byte load; the second buffer's start only for the rare
         // tuples past a buffer boundary
-        const uint32_t b = bucket_of(part_hash<KW, IDENT>(y.k), bf);
+        const uint32_t b = bucket_of(part_hash<KW, IDENT || STORE_H>(y.k), bf);
         const uint2 v = s_dlsp[b];
         return (i < v.y ? v.x : s_dl2[b]) + i;
-      } else return s_dl[bucket_of(part_hash<KW, IDENT>(y.k), bf)] + i;
+      } else return s_dl[bucket_of(part_hash<KW, IDENT || STORE_H>(y.k), bf)] + i;
     };
     if constexpr (PEER) {
       auto put = [&](uint32_t i) {
         const Tp y = s_tile[i];
-        const uint32_t b = bucket_of(part_hash<KW, IDENT>(y.k), bf);
+        const uint32_t b = bucket_of(part_hash<KW, IDENT || STORE_H>(y.k), bf);
         s_out[b][s_dl[b] + i] = y;
       };
       if (full) {
@@ -1776,10 +1809,11 @@ k_build_probe(JoinArgs a) {
 // unpack AoS tuples into key / payload columns (debug entry point only)
 template <int KW, int PW>
 __global__ void k_unpack(const Tup<KW, PW>* __restrict__ t, uint32_t n, typename UW<KW>::T* __restrict__ k,
-                         typename UW<PW>::T* __restrict__ p) {
+                         typename UW<PW>::T* __restrict__ p, uint32_t unmix) {
   for (uint32_t i = blockIdx.x * blockDim.x + threadIdx.x; i < n; i += gridDim.x * blockDim.x) {
     const Tup<KW, PW> x = t[i];
-    k[i] = x.k;
+    if constexpr (KW == 4) k[i] = unmix ? fmix32_inv(x.k) : x.k;
+    else k[i] = unmix ? fmix64_inv(x.k) : x.k;
     p[i] = x.v;
   }
 }
