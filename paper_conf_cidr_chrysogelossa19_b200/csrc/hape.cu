@@ -426,11 +426,12 @@ static hape_status launch_hist_joint(hape_join* h, int kw, const Src& s, SegMap 
   return HAPE_OK;
 }
 
-static hape_status launch_joint_reduce(hape_join* h, const uint16_t* part, uint32_t nparts, const uint32_t* ovf,
-                                       const uint32_t* rowsum, uint32_t P1, uint32_t P2, uint32_t* bounds1,
-                                       uint32_t* cursor1, uint32_t* bounds2, uint32_t* cursor2) {
-  k_joint_reduce<<<P1, JR_THREADS, 0, h->stream>>>(part, nparts, ovf, rowsum, P1, P2, bounds1, cursor1, bounds2,
-                                                   cursor2);
+// nrel relations' joint reductions in one launch (grid.y = relation: R's
+// and S's 2 x 256-row reductions fill the GPU together, C2 2 x 24 us -> one)
+static hape_status launch_joint_reduce(hape_join* h, const JrArgs* a, int nrel, uint32_t P1, uint32_t P2) {
+  JrArgs2 args{};
+  for (int i = 0; i < nrel; i++) args.r[i] = a[i];
+  k_joint_reduce<<<dim3(P1, (unsigned)nrel), JR_THREADS, 0, h->stream>>>(args, P1, P2);
   CK_LAUNCH(h);
   return HAPE_OK;
 }
@@ -917,12 +918,17 @@ static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const
     return launch_hist(h, kw, io[s].in, m1[s], bf1, P1, claim ? nullptr : at<uint32_t>(h, L.side[s].hist1),
                        at<uint32_t>(h, L.side[s].rowsum1));
   };
+  auto jr_args = [&](int s) {
+    return JrArgs{at<uint16_t>(h, L.side[s].part), L.side[s].nparts, at<uint32_t>(h, L.side[s].rowsum2),
+                  at<uint32_t>(h, L.side[s].rowsum1), at<uint32_t>(h, L.side[s].bounds1),
+                  at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].bounds2),
+                  at<uint32_t>(h, L.side[s].hist2)};
+  };
   auto scan1 = [&](int s) {
-    if (joint)
-      return launch_joint_reduce(h, at<uint16_t>(h, L.side[s].part), L.side[s].nparts,
-                                 at<uint32_t>(h, L.side[s].rowsum2), at<uint32_t>(h, L.side[s].rowsum1), P1, P2,
-                                 at<uint32_t>(h, L.side[s].bounds1), at<uint32_t>(h, L.side[s].hist1),
-                                 at<uint32_t>(h, L.side[s].bounds2), at<uint32_t>(h, L.side[s].hist2));
+    if (joint) {
+      const JrArgs a = jr_args(s);
+      return launch_joint_reduce(h, &a, 1, P1, P2);
+    }
     if (claim) return totals_scan(m1[s], P1, L.side[s].hist1, L.side[s].rowsum1, L.side[s].bounds1);
     return launch_scan(h, m1[s], P1, at<uint32_t>(h, L.side[s].hist1), at<uint32_t>(h, L.side[s].rowsum1),
                        at<uint32_t>(h, L.side[s].bounds1));
@@ -995,7 +1001,12 @@ static hape_status run_partition_stages(hape_join* h, const hape_plan& pl, const
     mark(h, HAPE_STAGE_HIST1);
     for (int s = 0; s < nside; s++) CKS(hist1(s));
     mark(h, HAPE_STAGE_SCAN1);
-    for (int s = 0; s < nside; s++) CKS(scan1(s));
+    if (joint && nside == 2) {
+      const JrArgs a[2] = {jr_args(0), jr_args(1)};
+      CKS(launch_joint_reduce(h, a, 2, P1, P2));
+    } else {
+      for (int s = 0; s < nside; s++) CKS(scan1(s));
+    }
     mark(h, HAPE_STAGE_SCATTER1);
     for (int s = 0; s < nside; s++) CKS(scatter1(s));
     if (pl.passes == 2) {

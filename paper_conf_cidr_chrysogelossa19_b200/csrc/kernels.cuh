@@ -655,10 +655,25 @@ k_hist_joint(PartIn in, SegMap m, uint32_t P1, uint32_t P2, uint32_t* __restrict
 // both passes.  P2/2 words per row; thread groups split the partial index.
 constexpr int JR_THREADS = 512;  // (1024 threads, 8 groups per row: measured +0.1 ms per C2 step)
 
+// one relation's joint-reduce arguments; blockIdx.y picks the relation, so
+// R's and S's reductions run as one launch
+struct JrArgs {
+  const uint16_t* part; uint32_t nparts; const uint32_t* ovf; const uint32_t* rowsum;
+  uint32_t* bounds1; uint32_t* cursor1; uint32_t* bounds2; uint32_t* cursor2;
+};
+struct JrArgs2 { JrArgs r[2]; };
+
 __global__ void __launch_bounds__(JR_THREADS)
-k_joint_reduce(const uint16_t* __restrict__ part, uint32_t nparts, const uint32_t* __restrict__ ovf,
-               const uint32_t* __restrict__ rowsum, uint32_t P1, uint32_t P2, uint32_t* __restrict__ bounds1,
-               uint32_t* __restrict__ cursor1, uint32_t* __restrict__ bounds2, uint32_t* __restrict__ cursor2) {
+k_joint_reduce(JrArgs2 args, uint32_t P1, uint32_t P2) {
+  const JrArgs& A = args.r[blockIdx.y];
+  const uint16_t* __restrict__ part = A.part;
+  const uint32_t nparts = A.nparts;
+  const uint32_t* __restrict__ ovf = A.ovf;
+  const uint32_t* __restrict__ rowsum = A.rowsum;
+  uint32_t* __restrict__ bounds1 = A.bounds1;
+  uint32_t* __restrict__ cursor1 = A.cursor1;
+  uint32_t* __restrict__ bounds2 = A.bounds2;
+  uint32_t* __restrict__ cursor2 = A.cursor2;
   __shared__ uint32_t row[4096];
   __shared__ uint32_t wtmp[33];
   __shared__ uint32_t s_b0;
