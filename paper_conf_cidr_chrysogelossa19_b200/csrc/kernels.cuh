@@ -1115,8 +1115,9 @@ k_scatter(PartIn in, SegMap m, BitField bf, uint32_t P, uint32_t* __restrict__ o
     asm volatile("fence.proxy.async.shared::cta;" ::: "memory");
     __syncthreads();  // C: the reordered tile is complete
     // phase 4: write the runs; consecutive threads -> consecutive addresses
-    // (the bucket is recomputed from the key: ALU is cheaper than another
-    // random shared-memory store + load)
+    // (the bucket is taken again from the tuple's h(k) -- stored in phase 1,
+    // STORE_H -- which is cheaper than another random shared-memory store +
+    // load)
     auto dst_of = [&](uint32_t i, const Tp& y) -> uint32_t {
       if constexpr (C::DST) return s_dst[i];
       else if constexpr (LINKED) {
