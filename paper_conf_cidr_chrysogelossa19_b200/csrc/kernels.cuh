@@ -1535,7 +1535,9 @@ __device__ __forceinline__ void jn_probe_batch(const JnTable<KW, PRW, LAY>& t, c
 // are register-budgeted for; A/B builds)
 #ifndef HAPE_JN_MINB
 // the direct form (8-byte S tuples, no pairs) at 4 CTAs per SM: <= 56
-// registers, no spills; unbounded it took 63 (3 CTAs per SM: C2 0.78 vs 0.74 ms)
+// registers, no spills; unbounded it took 63 (3 CTAs per SM: C2 0.78 vs 0.74 ms).
+// 5 CTAs per SM compiles to 40 registers without spills since the batch
+// changes, but measured no faster (C2 0.638 vs 0.633 ms, bag 0.910 vs 0.841)
 #define HAPE_JN_MINB 4
 #endif
 #ifndef HAPE_JN_SR_MINB
