@@ -701,10 +701,12 @@ static hape_status launch_join_m(hape_join* h, const JoinArgs& a, bool mat, uint
   // 2^28-tuple relations, C4's share at N = 8) run 512 consumer threads at 2
   // CTAs per SM with a 2^13-slot table, where the 256-thread form drops to 3
   // CTAs per SM at load factor 1 (C4/8 build+probe 1.466 -> 1.215 ms, 0.45 ->
-  // 0.54 of HBM); 2 K-tuple co-partitions stay on 256 (C2 0.643 vs 0.664 ms).
+  // 0.54 of HBM); so do probe-heavy joins (|S| >= 2|R|: C5's 4 S tuples per R
+  // tuple, 3.82 -> 3.36 ms), where more probes share each build; 2 K-tuple
+  // co-partitions with |S| = |R| stay on 256 (C2 0.643 vs 0.664 ms).
   // HAPE_JN_NC=256/512 forces the shape (A/B)
   static const int nc_env = env_int("HAPE_JN_NC", 0);
-  if (KW + PSW <= 8 && (nc_env == 512 || (nc_env == 0 && a.cap > 3072)))
+  if (KW + PSW <= 8 && (nc_env == 512 || (nc_env == 0 && (a.cap > 3072 || a.probe_heavy))))
     return launch_join_t<KW, PRW, PSW, false, 0, 512>(h, a, ctas);
   return launch_join_t<KW, PRW, PSW, false, 0, 256>(h, a, ctas);
 }
@@ -1414,6 +1416,7 @@ static hape_status local_join(hape_join* h, const Src loc_in[2], const MatOut& m
     // larger slices would thrash L2 a stage ahead of their use)
     static const int pf_env = [] { const char* e = getenv("HAPE_JN_PF"); return e ? atoi(e) : -1; }();
     ja.pf_bytes = pf_env >= 0 ? (uint32_t)pf_env : 32768u;
+    ja.probe_heavy = n_loc[1] >= 2 * n_loc[0] ? 1u : 0u;
     CKS(launch_join(h, kw, prw, psw, ja, mo.on, &pl.join_ctas));
     mark(h, HAPE_STAGE_FINALIZE);
     // local result: acc[4], out_ctr, ctrs

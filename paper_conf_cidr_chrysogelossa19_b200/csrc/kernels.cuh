@@ -1295,6 +1295,7 @@ struct JoinArgs {
   uint32_t nsb;                              // SR kernels: staged S tiles in the ring (>= 2)
   uint32_t qmask;                            // co-partitions - 1: q = h(key) & qmask (k_join_oa)
   uint32_t ep_period;                        // chain-head epochs before a head reset (<= 65535)
+  uint32_t probe_heavy;                      // host-side shape hint: |S| >= 2|R| (kernels ignore it)
 };
 
 struct JnStage {
