@@ -482,7 +482,9 @@ def main():
             # §8.d.3): one NCCL all-to-all of the same bytes per rank, CUDA
             # events on this stream, max over ranks
             try:
-                buf = torch.empty(xb // 4 // world * world, dtype=torch.int32, device="cuda")
+                # the same size on every rank (ragged shards differ by a row)
+                per = t * (n_r + n_s) // world
+                buf = torch.empty(per // 4 // world * world, dtype=torch.int32, device="cuda")
                 out = torch.empty_like(buf)
                 for _ in range(2):
                     dist.all_to_all_single(out, buf)
