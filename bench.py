@@ -481,11 +481,20 @@ def main():
             # the NVLink reference the exchange stage is read against (SURVEY
             # §8.d.3): one NCCL all-to-all of the same bytes per rank, CUDA
             # events on this stream, max over ranks
+            buf = out = None
             try:
                 # the same size on every rank (ragged shards differ by a row)
                 per = t * (n_r + n_s) // world
                 buf = torch.empty(per // 4 // world * world, dtype=torch.int32, device="cuda")
                 out = torch.empty_like(buf)
+            except Exception:
+                buf = out = None
+            # every rank runs the collective, or none does
+            okf = torch.tensor([1 if buf is not None else 0], dtype=torch.int32, device="cuda")
+            dist.all_reduce(okf, op=dist.ReduceOp.MIN)
+            try:
+                if int(okf.item()) != 1:
+                    raise RuntimeError("all-to-all reference buffers not allocated on every rank")
                 for _ in range(2):
                     dist.all_to_all_single(out, buf)
                 barrier()
